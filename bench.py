@@ -1,0 +1,468 @@
+#!/usr/bin/env python
+"""Benchmark of the perforated stencil hot path (BASELINE.json metric:
+Mpixel/s and speedup vs the exact kernel at the stated mean relative error;
+HBM GB/s).
+
+Default workload (N=1): BASELINE configs[1] (C2) -- Gaussian 5x5 fp32 on
+4096x4096 synthetic "natural" frames, row perforation, skipped fraction 1/2,
+linear-interpolation reconstruction (the paper's Rows1:LI).  A step is one
+perf_run over a batch of BATCH frames (512 MiB in + 512 MiB out, > L2, so no
+flush is needed between steps).  The remaining C2 variants (Gaussian5 and
+Sobel3 x row/col/checker x NN/LI x skipped 1/2, 1/4, 3/4) are timed the same
+way after the headline and reported under "variants".
+
+  python bench.py [--gpus N] [--steps K] [--warmup W] [--config C2|C1|C3|C4|C5] [--impl reference]
+
+Under torchrun each rank runs its own batch (weak scaling, no data-path
+collective); the timed region is bracketed by barriers + synchronize and the
+max over ranks is reported.  --impl reference times the CPU oracle (the
+paper-derived reference of this tier) on a bounded sample on rank 0.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import subprocess
+import sys
+import threading
+import time
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+METRIC = "Mpixel/s (and speedup vs exact kernel) at stated mean relative error; HBM GB/s"
+
+CONFIGS = {
+    "C1": dict(app="gaussian", r=2, W=512, H=512, batch=512, scheme="row", rate=(1, 2), recon="li",
+               cls="natural", seed=0x5EED0001, workload="C1: Gaussian 5x5 fp32 512x512, row 1/2, LI"),
+    "C2": dict(app="gaussian", r=2, W=4096, H=4096, batch=8, scheme="row", rate=(1, 2), recon="li",
+               cls="natural", seed=0x5EED0011,
+               workload="C2: Gaussian 5x5 fp32 4096x4096, row perforation 1/2, LI (headline of the C2 sweep)"),
+    "C3": dict(app="median", r=1, W=8192, H=8192, batch=4, scheme="col", rate=(1, 2), recon="nn",
+               cls="natural", seed=0x5EED0020, workload="C3: Median 3x3 u8 8192x8192, column perforation 1/2, NN"),
+    "C4": dict(app="hotspot", r=1, W=16384, H=16384, iters=200, scheme="row", rate=(1, 2), recon="li",
+               seed=0x5EED0030, workload="C4: Hotspot fp32 16384x16384, 200 iterations, row perforation 1/2, LI"),
+    "C5": dict(app="gauss_sobel", r=2, W=3840, H=2160, batch=16, scheme="row", rate=(1, 2), recon="li",
+               cls="natural", seed=0x5EED1000,
+               workload="C5: Gaussian5->Sobel3 fp32 3840x2160 frames, row perforation 1/2, LI"),
+}
+
+
+def kept_fraction(scheme, rate):
+    num, den = rate
+    return 1.0 if scheme == "none" or num == 0 else 1.0 - num / den
+
+
+def bytes_per_px(app, scheme, rate):
+    """algorithmic bytes per output pixel: kept input + full output (DESIGN.md Roofline)"""
+    k = kept_fraction(scheme, rate)
+    if app == "median":
+        return k * 1 + 1
+    if app == "hotspot":
+        return k * 8 + 4  # T and P kept, T' written
+    return k * 4 + 4
+
+
+def load_peaks():
+    p = os.path.join(ROOT, "MEASURED_PEAKS.json")
+    if os.path.exists(p):
+        d = json.load(open(p))
+        return float(d["hbm_gbs"]), "measured (MEASURED_PEAKS.json copy)"
+    return 6650.0, "fallback (B200_PROFILING.md)"
+
+
+def ncu_traffic(kernel_key):
+    """per-launch DRAM bytes from a committed ncu --set full capture, if present"""
+    p = os.path.join(ROOT, "profiles", "ncu_traffic.json")
+    if not os.path.exists(p):
+        return None
+    try:
+        return json.load(open(p)).get(kernel_key)
+    except Exception:
+        return None
+
+
+class ClockSampler:
+    FIELDS = ("clocks.sm,clocks.max.sm,power.draw,clocks_event_reasons.hw_slowdown,"
+              "clocks_event_reasons.hw_thermal_slowdown,clocks_event_reasons.sw_thermal_slowdown,"
+              "clocks_event_reasons.sw_power_cap")
+
+    def __init__(self, index):
+        self.index = index
+        self.rows = []
+        self.proc = None
+
+    def __enter__(self):
+        try:
+            self.proc = subprocess.Popen(
+                ["nvidia-smi", "-i", str(self.index), f"--query-gpu={self.FIELDS}", "--format=csv,noheader,nounits",
+                 "-lms", "100"], stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
+            self.t = threading.Thread(target=self._read, daemon=True)
+            self.t.start()
+            time.sleep(0.3)
+        except Exception:
+            self.proc = None
+        return self
+
+    def _read(self):
+        for line in self.proc.stdout:
+            parts = [x.strip() for x in line.split(",")]
+            if len(parts) >= 7:
+                self.rows.append(parts)
+
+    def __exit__(self, *a):
+        if self.proc:
+            self.proc.terminate()
+            try:
+                self.proc.wait(timeout=2)
+            except Exception:
+                self.proc.kill()
+
+    def summary(self):
+        if not self.rows:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["unsampled"]}
+        sm = [float(r[0]) for r in self.rows if r[0].replace(".", "").isdigit()]
+        mx = [float(r[1]) for r in self.rows if r[1].replace(".", "").isdigit()]
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        reasons = sorted({names[i] for r in self.rows for i in range(4) if r[3 + i].lower() == "active"})
+        return {"sm_mhz": statistics.median(sm) if sm else None, "sm_max_mhz": max(mx) if mx else None,
+                "reasons": reasons, "samples": len(self.rows)}
+
+
+def dist_setup(args):
+    import torch
+    ws = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    if ws > 1:
+        import torch.distributed as dist
+        os.environ.setdefault("MASTER_ADDR", "127.0.0.1")
+        torch.cuda.set_device(local)
+        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+    else:
+        torch.cuda.set_device(0)
+    return ws, rank, local
+
+
+def barrier(ws):
+    if ws > 1:
+        import torch.distributed as dist
+        dist.barrier()
+
+
+def max_over_ranks(ws, v):
+    if ws == 1:
+        return v
+    import torch
+    import torch.distributed as dist
+    t = torch.tensor([v], dtype=torch.float64, device="cuda")
+    dist.all_reduce(t, op=dist.ReduceOp.MAX)
+    return float(t.item())
+
+
+def time_kernel(fn, stream, reps, warm):
+    """average device time per call (ms), CUDA events on the launching stream"""
+    import torch
+    for _ in range(warm):
+        fn()
+    torch.cuda.synchronize()
+    a = torch.cuda.Event(enable_timing=True)
+    b = torch.cuda.Event(enable_timing=True)
+    a.record(stream)
+    for _ in range(reps):
+        fn()
+    b.record(stream)
+    b.synchronize()
+    return a.elapsed_time(b) / reps
+
+
+# ---------------------------------------------------------------------------
+def oracle_sample(cfg, rows=256):
+    """time the oracle (as it stands, single-threaded) on a bounded sample:
+    the first `rows` rows of one frame of the config (fresh image each call)."""
+    import oracle
+    import synth
+    app, W = cfg["app"], cfg["W"]
+    if app == "hotspot":
+        n = min(cfg["W"], 1024)
+        T, P = synth.hotspot(cfg["seed"], n, rows)
+        prm = oracle.params("hotspot", n, rows, 1, cfg["scheme"], cfg["rate"], cfg["recon"])
+        t0 = time.perf_counter()
+        oracle.hotspot(prm, T, P, 1)
+        return (n * rows) / (time.perf_counter() - t0), f"1 Hotspot step on a {n}x{rows} grid"
+    u8 = app == "median"
+    img = synth.image(cfg["cls"], cfg["seed"], W, rows, np.uint8 if u8 else np.float32)
+    prm = oracle.params(app, W, rows, cfg["r"], cfg["scheme"], cfg["rate"], cfg["recon"], 32 if u8 else 8)
+    t0 = time.perf_counter()
+    oracle.run(prm, img)
+    return (W * rows) / (time.perf_counter() - t0), f"{W}x{rows} rows of one frame"
+
+
+def cpu_baseline(cfg, budget_s=10.0):
+    px = 0.0
+    t = 0.0
+    n = 0
+    desc = ""
+    while t < budget_s and n < 200:
+        rate, desc = oracle_sample(cfg)
+        # rate = px/s for this call; accumulate time-weighted
+        dt = None
+        px_call = cfg["W"] * 256 if cfg["app"] != "hotspot" else min(cfg["W"], 1024) * 256
+        dt = px_call / rate
+        px += px_call
+        t += dt
+        n += 1
+    return {"value": px / t / 1e6, "unit": "Mpixel/s" if cfg["app"] != "hotspot" else "Mcell-updates/s",
+            "cores": 1, "kind": "oracle", "sample": f"{n} x oracle.run on {desc} ({t:.1f} s of CPU work)"}
+
+
+def run_reference(args, ws, rank):
+    cfg = CONFIGS[args.config]
+    if rank != 0:
+        return
+    unit = "Mpixel/s" if cfg["app"] != "hotspot" else "Mcell-updates/s"
+    for _ in range(args.warmup):
+        oracle_sample(cfg)
+    rates, t_total, px_total = [], 0.0, 0
+    for _ in range(args.steps):
+        r, desc = oracle_sample(cfg)
+        px = cfg["W"] * 256 if cfg["app"] != "hotspot" else min(cfg["W"], 1024) * 256
+        t_total += px / r
+        px_total += px
+    v = px_total / t_total / 1e6
+    line = {"impl": "reference", "metric": METRIC, "value": v, "unit": unit, "n_gpus": args.gpus,
+            "steps": args.steps, "warmup": args.warmup, "ms_per_step": 1e3 * t_total / args.steps,
+            "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "f64", "data": "synthetic",
+            "config": {"workload": cfg["workload"], "sample": f"each step: oracle.run on {desc}"},
+            "cpu_baseline": {"value": v, "unit": unit, "cores": 1, "kind": "oracle",
+                             "sample": f"{args.steps} steps of oracle.run on {desc}"},
+            "e2e": {"value": v, "unit": unit, "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
+    print(json.dumps(line), flush=True)
+
+
+# ---------------------------------------------------------------------------
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=20)
+    ap.add_argument("--warmup", type=int, default=5)
+    ap.add_argument("--config", default="C2", choices=sorted(CONFIGS))
+    ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
+    ap.add_argument("--no-variants", action="store_true")
+    ap.add_argument("--no-cpu", action="store_true")
+    ap.add_argument("--batch", type=int, default=0)
+    args = ap.parse_args()
+    args.warmup = max(args.warmup, 3)
+
+    if args.impl == "reference":
+        ws = int(os.environ.get("WORLD_SIZE", "1"))
+        rank = int(os.environ.get("RANK", "0"))
+        run_reference(args, ws, rank)
+        return
+
+    import torch
+
+    import paper_conf_cgo_maiercj18_b200 as kp
+    import synth
+
+    ws, rank, local = dist_setup(args)
+    cfg = dict(CONFIGS[args.config])
+    if args.batch:
+        cfg["batch"] = args.batch
+    stream = torch.cuda.current_stream()
+    peak, peak_src = load_peaks()
+    app, W, H = cfg["app"], cfg["W"], cfg["H"]
+    u8 = app == "median"
+    es = 1 if u8 else 4
+    unit = "Mpixel/s" if app != "hotspot" else "Mcell-updates/s"
+
+    if app == "hotspot":
+        result = bench_hotspot(args, cfg, ws, rank, local, stream, peak, peak_src)
+    else:
+        B = cfg["batch"]
+        dt = torch.uint8 if u8 else torch.float32
+        x = torch.empty((B, H, W), dtype=dt, device="cuda")
+        # per-rank distinct frames: seed + rank * B + f
+        synth.image_device(cfg["cls"], cfg["seed"] + rank * B, W, H, B, x.data_ptr(), u8, stream.cuda_stream)
+        y = torch.empty_like(x)
+        yex = torch.empty_like(x)
+        G = 32 if u8 else 32
+        plan = kp.Plan(app, W, H, cfg["r"], cfg["scheme"], cfg["rate"], cfg["recon"], batch=B, granule_bytes=G)
+        exact = kp.Plan(app, W, H, cfg["r"], "none", (0, 1), "nn", batch=B)
+        run = lambda: plan.run(x, y, stream)  # noqa: E731
+        for _ in range(args.warmup):
+            run()
+        torch.cuda.synchronize()
+        barrier(ws)
+        torch.cuda.synchronize()
+        with ClockSampler(local) as clk:
+            e0 = torch.cuda.Event(enable_timing=True)
+            e1 = torch.cuda.Event(enable_timing=True)
+            e0.record(stream)
+            for _ in range(args.steps):
+                run()
+            e1.record(stream)
+            e1.synchronize()
+        torch.cuda.synchronize()
+        barrier(ws)
+        ms = max_over_ranks(ws, e0.elapsed_time(e1) / args.steps)
+        px_step = B * W * H
+        value = ws * px_step / (ms * 1e-3) / 1e6
+        # exact kernel, same batch (speedup) and error at the stated MRE
+        ms_exact = max_over_ranks(ws, time_kernel(lambda: exact.run(x, yex, stream), stream, args.steps,
+                                                  args.warmup))
+        mre, cnt = plan.error(yex, y, stream)
+        algo_b = bytes_per_px(app, cfg["scheme"], cfg["rate"]) * px_step
+        achieved = algo_b / (ms * 1e-3) / 1e9
+        kkey = f"{app}{cfg['r']}_{cfg['scheme']}_{cfg['rate'][0]}-{cfg['rate'][1]}_{cfg['recon']}"
+        tr = ncu_traffic(kkey)
+        result = {
+            "metric": METRIC, "value": value, "unit": unit, "n_gpus": ws, "steps": args.steps,
+            "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True, "scaling": "weak",
+            "vs_baseline": None, "dtype": "u8" if u8 else "f32", "data": "synthetic",
+            "config": {"workload": cfg["workload"], "W": W, "H": H, "frames_per_gpu": B,
+                       "granule_bytes": G, "l2": "inputs larger than L2 (batch of frames, no flush)",
+                       "parallelism": f"frames sharded, {B} per GPU" if ws > 1 else "single GPU"},
+            "speedup_vs_exact": ms_exact / ms, "exact_ms_per_step": ms_exact,
+            "exact_mpixel_s": ws * px_step / (ms_exact * 1e-3) / 1e6,
+            "error": {"metric": "mre" if app not in ("sobel", "gauss_sobel") else "me", "value": mre,
+                      "count": cnt},
+            "hbm_gbs": achieved,
+            "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
+                         "frac": achieved / peak, "traffic": tr, "kernel": kkey,
+                         "algorithmic_bytes_per_launch": algo_b, "peak_source": peak_src},
+            "clocks": clk.summary(),
+            "gpu_launches": args.steps,
+        }
+        # e2e through the C ABI with pinned host buffers (one frame per step)
+        result["e2e"] = bench_e2e(kp, cfg, stream, args, ws, x)
+        if not args.no_variants and args.config == "C2":
+            result["variants"] = bench_variants(kp, cfg, x, y, yex, stream, peak, ws)
+        plan.close()
+        exact.close()
+    if rank == 0 and not args.no_cpu:
+        result["cpu_baseline"] = cpu_baseline(cfg)
+    if rank == 0:
+        print(json.dumps(result), flush=True)
+    if ws > 1:
+        import torch.distributed as dist
+        dist.destroy_process_group()
+
+
+def bench_e2e(kp, cfg, stream, args, ws, x):
+    import torch
+    app, W, H = cfg["app"], cfg["W"], cfg["H"]
+    u8 = app == "median"
+    hin = x[0].cpu().pin_memory()
+    hout = torch.empty_like(hin).pin_memory()
+    plan = kp.Plan(app, W, H, cfg["r"], cfg["scheme"], cfg["rate"], cfg["recon"], batch=1)
+    f = lambda: plan.run_host(hin, hout, stream)  # noqa: E731
+    for _ in range(3):
+        f()
+    torch.cuda.synchronize()
+    barrier(ws)
+    steps = max(3, min(args.steps, 10))
+    e0 = torch.cuda.Event(enable_timing=True)
+    e1 = torch.cuda.Event(enable_timing=True)
+    e0.record(stream)
+    for _ in range(steps):
+        f()
+    e1.record(stream)
+    e1.synchronize()
+    ms = max_over_ranks(ws, e0.elapsed_time(e1) / steps)
+    plan.close()
+    nb = W * H * (1 if u8 else 4)
+    return {"value": ws * W * H / (ms * 1e-3) / 1e6, "unit": "Mpixel/s" if app != "hotspot" else "Mcell-updates/s",
+            "h2d_bytes_per_step": nb, "d2h_bytes_per_step": nb, "ms_per_step": ms,
+            "api": "perf_run_host (pinned host buffers, one frame per step)"}
+
+
+def bench_variants(kp, cfg, x, y, yex, stream, peak, ws):
+    W, H, B = cfg["W"], cfg["H"], cfg["batch"]
+    px = B * W * H
+    out = []
+    for app, r in (("gaussian", 2), ("sobel", 1)):
+        ex = kp.Plan(app, W, H, r, "none", (0, 1), "nn", batch=B)
+        ms_ex = time_kernel(lambda: ex.run(x, yex, stream), stream, 10, 3)
+        out.append({"app": app, "r": r, "scheme": "none", "rate": [0, 1], "recon": "-", "ms": ms_ex,
+                    "mpixel_s": px / ms_ex / 1e3, "speedup": 1.0, "error": 0.0,
+                    "hbm_gbs": 8 * px / ms_ex / 1e6, "frac": 8 * px / ms_ex / 1e6 / peak})
+        for scheme in ("row", "col", "checker"):
+            for rate in ((1, 2), (1, 4), (3, 4)):
+                for recon in ("nn", "li"):
+                    p = kp.Plan(app, W, H, r, scheme, rate, recon, batch=B)
+                    ms = time_kernel(lambda: p.run(x, y, stream), stream, 10, 3)
+                    err, _ = p.error(yex, y, stream)
+                    gbs = bytes_per_px(app, scheme, rate) * px / ms / 1e6
+                    out.append({"app": app, "r": r, "scheme": scheme, "rate": list(rate), "recon": recon,
+                                "ms": ms, "mpixel_s": px / ms / 1e3, "speedup": ms_ex / ms, "error": err,
+                                "hbm_gbs": gbs, "frac": gbs / peak,
+                                "ceiling": (8.0) / bytes_per_px(app, scheme, rate)})
+                    p.close()
+        ex.close()
+    return out
+
+
+def bench_hotspot(args, cfg, ws, rank, local, stream, peak, peak_src):
+    import torch
+
+    import paper_conf_cgo_maiercj18_b200 as kp
+    import synth
+    W, Hg, iters = cfg["W"], cfg["H"], cfg["iters"]
+    # row bands: rank k owns rows [y0, y0 + h)
+    cuts = [Hg * i // ws for i in range(ws + 1)]
+    y0, h = cuts[rank], cuts[rank + 1] - cuts[rank]
+    T = torch.empty((h, W), device="cuda")
+    P = torch.empty((h, W), device="cuda")
+    synth.hotspot_band_device(cfg["seed"], W, Hg, y0, h, T.data_ptr(), P.data_ptr(), stream.cuda_stream)
+    out = torch.empty_like(T)
+    keys = dict(iters=iters)
+    if ws > 1:
+        keys.update(global_h=Hg, band_y0=y0)
+    plan = kp.Plan("hotspot", W, h, 1, cfg["scheme"], cfg["rate"], cfg["recon"], **keys)
+    exact = kp.Plan("hotspot", W, h, 1, "none", (0, 1), "nn", **keys)
+    if ws > 1:
+        import torch.distributed as dist
+        uid = kp.perf_comm_unique_id() if rank == 0 else bytes(128)
+        t = torch.tensor(list(uid), dtype=torch.uint8, device="cuda")
+        dist.broadcast(t, 0)
+        uid = bytes(t.cpu().tolist())
+        kp.perf_comm_init(plan.handle, uid, rank, ws)
+        kp.perf_comm_init(exact.handle, uid, rank, ws)
+    run = lambda: plan.hotspot(T, P, out, stream)  # noqa: E731
+    run()
+    torch.cuda.synchronize()
+    barrier(ws)
+    with ClockSampler(local) as clk:
+        e0 = torch.cuda.Event(enable_timing=True)
+        e1 = torch.cuda.Event(enable_timing=True)
+        e0.record(stream)
+        for _ in range(args.steps):
+            run()
+        e1.record(stream)
+        e1.synchronize()
+    barrier(ws)
+    ms = max_over_ranks(ws, e0.elapsed_time(e1) / args.steps)
+    out_ex = torch.empty_like(T)
+    ms_ex = max_over_ranks(ws, time_kernel(lambda: exact.hotspot(T, P, out_ex, stream), stream, 2, 1))
+    mre, cnt = plan.error(out_ex, out, stream)
+    cells = W * Hg * iters
+    algo_b = bytes_per_px("hotspot", cfg["scheme"], cfg["rate"]) * W * h * iters
+    achieved = algo_b / (ms * 1e-3) / 1e9
+    return {"metric": METRIC, "value": cells / (ms * 1e-3) / 1e6, "unit": "Mcell-updates/s", "n_gpus": ws,
+            "steps": args.steps, "warmup": 1, "ms_per_step": ms, "higher_is_better": True,
+            "scaling": "strong", "vs_baseline": None, "dtype": "f32", "data": "synthetic",
+            "config": {"workload": cfg["workload"], "bands": ws, "halo": "NCCL send/recv per step" if ws > 1
+                       else "none"},
+            "speedup_vs_exact": ms_ex / ms, "error": {"metric": "mre", "value": mre, "count": cnt},
+            "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
+                         "frac": achieved / peak, "traffic": None, "peak_source": peak_src},
+            "clocks": clk.summary(), "gpu_launches": args.steps * iters}
+
+
+if __name__ == "__main__":
+    main()

@@ -1,0 +1,152 @@
+/*
+ * kperf.h -- C ABI of the B200-native hot path of local memory-aware kernel
+ * perforation (Maier, Cosenza, Juurlink, CGO'18; PAPER.md = the paper text).
+ *
+ * The paper states the problem as "input buffer -> data perforation -> data
+ * reconstruction -> kernel execution -> output buffer" (Fig. 1b,
+ * PAPER.md:258-274) with the perforation scheme, the reconstruction technique,
+ * the perforation rate and the work-group size as parameters (Sec. 6.3,
+ * PAPER.md:808-852).  Every entry point below is extern "C", takes plain
+ * pointers and sizes, returns a perf_status (PERF_OK = 0) and never throws.
+ * On failure perf_last_error() returns a thread-local message.
+ *
+ * Data layout: row-major, dense, pitch = W * sizeof(T); a batch of BATCH
+ * frames is frame-major (frame f starts at element f * W * H).  T is uint8_t
+ * for PERF_APP_MEDIAN and float for every other app.  Pixel (x, y) is element
+ * y * W + x.
+ *
+ * Ownership: the caller owns every buffer it passes (device buffers for the
+ * perf_run* calls, host buffers for perf_run_host) and keeps them alive until
+ * the work on `stream` completes.  A plan owns only scratch (error partials,
+ * Hotspot ping-pong/halo rows, staging buffers of perf_run_host).  `in` and
+ * `out` must not alias.  A plan is used by one stream at a time.  `stream` is
+ * a cudaStream_t (NULL = legacy default stream).
+ *
+ * Asynchrony: perf_run and perf_run_hotspot only enqueue work (asynchronous
+ * faults surface at the next synchronising call); perf_error and
+ * perf_run_host synchronise `stream` before returning.
+ */
+#ifndef KPERF_H
+#define KPERF_H
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+typedef enum {
+  PERF_OK = 0,
+  PERF_ERR_INVALID_ARG = 1, /* null pointer, bad size/enum/rate/radius, misuse */
+  PERF_ERR_UNSUPPORTED = 2, /* a combination the build does not provide */
+  PERF_ERR_CUDA = 3,        /* a CUDA runtime error (message in perf_last_error) */
+  PERF_ERR_NCCL = 4,        /* an NCCL error (sharded Hotspot) */
+  PERF_ERR_OOM = 5          /* scratch allocation failed */
+} perf_status;
+
+/* Applications of Sec. 6.1 (Table 1). */
+typedef enum {
+  PERF_APP_GAUSSIAN = 0,    /* binomial blur, radius 1 (3x3) or 2 (5x5), fp32 */
+  PERF_APP_SOBEL = 1,       /* gradient magnitude, radius 1 (3x3) or 2 (5x5), fp32 */
+  PERF_APP_MEDIAN = 2,      /* 3x3 median, radius 1, u8 */
+  PERF_APP_HOTSPOT = 3,     /* Rodinia 2D thermal step, radius 1, fp32 (perf_run_hotspot) */
+  PERF_APP_GAUSS_SOBEL = 4, /* Sobel3(Gaussian5(frame)), the C5 pipeline; radius must be 2 */
+  PERF_APP_INVERSION = 5    /* 255 - x, radius 0, fp32 */
+} perf_app;
+
+/* Perforation schemes (Sec. 4.4; Fig. 4). */
+typedef enum {
+  PERF_SCHEME_NONE = 0,    /* exact kernel: every input element is loaded */
+  PERF_SCHEME_ROW = 1,     /* skip whole rows; rebuilt along y */
+  PERF_SCHEME_COL = 2,     /* skip G-pixel column granules; rebuilt along x */
+  PERF_SCHEME_CHECKER = 3  /* skip G-pixel cells on a diagonal lattice; rebuilt along y */
+} perf_scheme;
+
+/* Reconstruction techniques (Sec. 5.1). */
+typedef enum {
+  PERF_RECON_NN = 0,     /* nearest loaded element; equidistant -> lower coordinate */
+  PERF_RECON_LINEAR = 1  /* linear interpolation; NN where one side is missing */
+} perf_recon;
+
+typedef enum {
+  PERF_METRIC_MRE = 0,   /* mean over {e != 0} of |e - a| / |e| */
+  PERF_METRIC_ME = 1,    /* sum |e - a| / sum |e|  (Sobel's "mean error", :580-584) */
+  PERF_METRIC_MAE = 2    /* mean |e - a| */
+} perf_metric;
+
+/* Skipped fraction num/den of the scheme's lines (rows, column granules or
+ * cells): num = 0 (exact), num = 1 (skip one line of every den: the line with
+ * phase den-1) or num = den-1 (keep one line of every den: phase 0).
+ * 1 <= den <= 8.  The paper's Rows1 = {1,2}, Rows2 = {3,4}. */
+typedef struct { int num, den; } perf_rate;
+
+typedef struct perf_plan_s* perf_plan_t;
+
+/* perf_plan_set keys.  None of them changes results except GRANULE_BYTES
+ * (the width G of a column/checker cell, part of the mask definition) and
+ * METRIC. */
+enum {
+  PERF_KEY_BATCH = 1,          /* frames per perf_run (default 1) */
+  PERF_KEY_ITERS = 2,          /* Hotspot steps per perf_run_hotspot (default 1) */
+  PERF_KEY_GRANULE_BYTES = 3,  /* G * sizeof(T) for COL/CHECKER (default 32; multiple of sizeof(T)) */
+  PERF_KEY_GLOBAL_H = 4,       /* sharded Hotspot: rows of the whole grid (default H) */
+  PERF_KEY_BAND_Y0 = 5,        /* sharded Hotspot: first global row of this rank's band (default 0) */
+  PERF_KEY_TILE_W = 6,         /* consumer warps per CTA (1..8); tile width = warps * 32 * V */
+  PERF_KEY_TILE_H = 7,         /* output rows per CTA segment (default 128) */
+  PERF_KEY_METRIC = 8,         /* perf_metric used by perf_error (default: MRE; ME for Sobel apps) */
+  PERF_KEY_LOADER = 9,         /* 0 auto, 1 TMA bulk rows, 2 cp.async 16 B, 3 scalar (any alignment) */
+  PERF_KEY_RING = 10           /* shared-memory ring depth in rows (0 = auto) */
+};
+
+/* Create a plan.  Validates: W, H >= 1; radius allowed for the app (Gaussian,
+ * Sobel {1,2}; Median, Hotspot {1}; Gauss-Sobel {2}; Inversion {0});
+ * den in [1,8], num in {0, 1, den-1}; CHECKER needs H >= den (every column
+ * must hold a loaded element).  No device work, no allocation on the device. */
+perf_status perf_plan(perf_plan_t* plan, perf_app app, int W, int H, int radius, perf_scheme scheme,
+                      perf_rate rate, perf_recon recon);
+perf_status perf_plan_set(perf_plan_t plan, int key, long long value);
+perf_status perf_plan_get(perf_plan_t plan, int key, long long* value);
+
+/* Run the fused perforated load -> rebuild -> stencil kernel over BATCH frames
+ * of device memory: in, out are device pointers to BATCH * W * H elements of T.
+ * Asynchronous on `stream`. */
+perf_status perf_run(perf_plan_t plan, const void* in, void* out, void* stream);
+
+/* Same computation on HOST buffers (pinned or pageable): copies in -> device,
+ * runs, copies out -> host, synchronises `stream`.  The plan owns the device
+ * staging buffers. */
+perf_status perf_run_host(perf_plan_t plan, const void* host_in, void* host_out, void* stream);
+
+/* ITERS Hotspot steps on device buffers of W * H floats (a band of H rows
+ * starting at global row BAND_Y0 of a GLOBAL_H-row grid when sharded).  T and
+ * P are both perforated and rebuilt every step.  temp_in is not modified. */
+perf_status perf_run_hotspot(perf_plan_t plan, const float* temp_in, const float* power, float* temp_out,
+                             void* stream);
+
+/* Single-device emulation of the sharded Hotspot (used by the tests): nb plans
+ * describing consecutive bands of one grid (GLOBAL_H, BAND_Y0 set, same ITERS)
+ * step in lockstep on `stream`; halo rows move by device copies instead of
+ * NCCL, through the same band buffers and kernels as perf_run_hotspot.
+ * temp_in, power, temp_out are whole-grid device buffers. */
+perf_status perf_run_hotspot_bands_local(perf_plan_t* plans, int nb, const float* temp_in, const float* power,
+                                         float* temp_out, void* stream);
+
+/* Error of `approx` against `exact` (device pointers, BATCH * W * H elements of
+ * the plan's T): the plan's metric in fp64, deterministic two-pass reduction.
+ * Writes the value and the count of contributing elements; synchronises. */
+perf_status perf_error(perf_plan_t plan, const void* exact, const void* approx, void* stream,
+                       double* err_out, long long* count_out);
+
+/* Sharded Hotspot: attach an NCCL communicator built from a 128-byte
+ * ncclUniqueId (rank, nranks).  Rank k holds global rows
+ * [BAND_Y0, BAND_Y0 + H); neighbours exchange loaded halo rows every step. */
+perf_status perf_comm_init(perf_plan_t plan, const void* nccl_unique_id, int rank, int nranks);
+/* Fill a 128-byte buffer with a fresh ncclUniqueId (rank 0 calls this). */
+perf_status perf_comm_unique_id(void* out_128_bytes);
+
+perf_status perf_destroy(perf_plan_t plan);
+const char* perf_last_error(void);
+const char* perf_version(void);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* KPERF_H */

@@ -1,0 +1,7 @@
+// k_gauss2.cu -- instantiations of the perforated stencil kernel for AppGauss<2>.
+#include "kernel.cuh"
+namespace kp {
+cudaError_t launch_gauss2(int scheme, int recon, const KParams& p, unsigned grid, size_t smem, cudaStream_t s) {
+  return launch_app<AppGauss<2>, kNCW>(scheme, recon, p, grid, smem, s);
+}
+}  // namespace kp

@@ -1,0 +1,7 @@
+// k_sobel1.cu -- instantiations of the perforated stencil kernel for AppSobel<1>.
+#include "kernel.cuh"
+namespace kp {
+cudaError_t launch_sobel1(int scheme, int recon, const KParams& p, unsigned grid, size_t smem, cudaStream_t s) {
+  return launch_app<AppSobel<1>, kNCW>(scheme, recon, p, grid, smem, s);
+}
+}  // namespace kp

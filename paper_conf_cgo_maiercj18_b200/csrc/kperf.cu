@@ -1,0 +1,557 @@
+// kperf.cu -- the C ABI (include/kperf.h): plan validation, launch geometry,
+// Hotspot time loop (single device, banded with NCCL halo exchange, or banded
+// on one device for testing), error metric, host-buffer entry point.
+#include <cuda_runtime.h>
+#include <nccl.h>
+
+#include <algorithm>
+#include <cstdio>
+#include <cstdlib>
+#include <cstring>
+#include <string>
+#include <vector>
+
+#include "../../include/kperf.h"
+#include "kernel.cuh"
+
+namespace kp {
+cudaError_t launch_error(int is_u8, const void* exact, const void* approx, long long n, int metric, double* scratch,
+                         cudaStream_t s);
+size_t error_scratch_doubles();
+}  // namespace kp
+
+using kp::KParams;
+
+static thread_local std::string g_err;
+
+static perf_status fail(perf_status st, const std::string& msg) {
+  g_err = msg;
+  return st;
+}
+static perf_status cuda_fail(cudaError_t e, const char* where) {
+  return fail(PERF_ERR_CUDA, std::string(where) + ": " + cudaGetErrorString(e));
+}
+#define CK(call)                                        \
+  do {                                                  \
+    cudaError_t e_ = (call);                            \
+    if (e_ != cudaSuccess) return cuda_fail(e_, #call); \
+  } while (0)
+
+struct Band {  // banded Hotspot state
+  int hb = 0;                 // halo rows each side
+  float* buf[2] = {nullptr, nullptr};
+  float* pbuf = nullptr;      // power with halo
+  size_t rows = 0;            // allocated rows (h + 2 hb)
+};
+
+struct perf_plan_s {
+  int app, W, H, radius, scheme, recon;
+  perf_rate rate;
+  long long batch = 1, iters = 1, granule_bytes = 32, global_h = -1, band_y0 = 0, tile_w = kp::kNCW, tile_h = 128,
+            metric = 0, loader = 0, ring = 0;
+  double* d_err = nullptr;
+  float* d_tmp = nullptr;
+  size_t tmp_elems = 0;
+  void* d_stage_in = nullptr;
+  void* d_stage_out = nullptr;
+  size_t stage_bytes = 0;
+  Band band;
+  ncclComm_t comm = nullptr;
+  int rank = 0, nranks = 1;
+};
+
+static size_t elem_size(int app) { return app == PERF_APP_MEDIAN ? 1 : 4; }
+
+static int next_pow2(int v) {
+  int p = 1;
+  while (p < v) p <<= 1;
+  return p;
+}
+static int log2i(int v) {
+  int l = 0;
+  while ((1 << l) < v) ++l;
+  return l;
+}
+
+// Launch geometry for rows [y_begin, y_end) of `frames` frames.
+static perf_status make_params(const perf_plan_s* P, const void* in, const void* in2, void* out, int frames,
+                               int in_row0, int avail0, int avail1, int out_row0, int y_begin, int y_end,
+                               KParams& k, unsigned& grid, size_t& smem) {
+  const int es = (int)elem_size(P->app);
+  const int V = 16 / es;
+  const int NCW = kp::kNCW;
+  const int TW = NCW * 32 * V;
+  const int Hg = P->global_h > 0 ? (int)P->global_h : P->H;
+  int scheme = P->scheme;
+  if (P->rate.num == 0) scheme = PERF_SCHEME_NONE;
+  std::memset(&k, 0, sizeof k);
+  k.in = in;
+  k.in2 = in2;
+  k.out = out;
+  k.in_fstride = (long long)P->W * P->H;
+  k.out_fstride = (long long)P->W * P->H;
+  k.W = P->W;
+  k.Hg = Hg;
+  k.in_row0 = in_row0;
+  k.avail0 = avail0;
+  k.avail1 = avail1;
+  k.out_row0 = out_row0;
+  k.y_begin = y_begin;
+  k.y_end = y_end;
+  k.num = scheme == PERF_SCHEME_NONE ? 0 : P->rate.num;
+  k.den = scheme == PERF_SCHEME_NONE ? 1 : P->rate.den;
+  k.keep_one = (k.num == k.den - 1) ? 1 : 0;
+  const int G = (int)(P->granule_bytes / es);
+  k.G = G < 1 ? 1 : G;
+  k.fast_ok = (scheme == PERF_SCHEME_NONE || scheme == PERF_SCHEME_ROW || (k.G % V) == 0) ? 1 : 0;
+  const bool aligned = ((reinterpret_cast<uintptr_t>(in) | reinterpret_cast<uintptr_t>(out) |
+                         reinterpret_cast<uintptr_t>(in2)) & 15) == 0;
+  k.vec_io = (P->W % V == 0) && aligned ? 1 : 0;
+  int loader = (int)P->loader;
+  if (loader == kp::L_AUTO) {
+    if (!k.vec_io) loader = kp::L_SCALAR;
+    else if (scheme == PERF_SCHEME_NONE || scheme == PERF_SCHEME_ROW) loader = kp::L_BULK;
+    else loader = k.fast_ok ? kp::L_ASYNC16 : kp::L_SCALAR;
+  }
+  if (loader == kp::L_BULK && !(k.vec_io && (scheme == PERF_SCHEME_NONE || scheme == PERF_SCHEME_ROW)))
+    return fail(PERF_ERR_UNSUPPORTED, "loader BULK needs the row/none scheme, W % V == 0 and 16-B aligned buffers");
+  if (loader == kp::L_ASYNC16 && !(k.vec_io && k.fast_ok))
+    return fail(PERF_ERR_UNSUPPORTED, "loader ASYNC16 needs W % V == 0, aligned buffers and G % V == 0");
+  k.loader = loader;
+  // halo / apron columns: the lane edge chunk (V) plus, for the column scheme,
+  // the distance to the nearest loaded granule on either side (<= den * G)
+  int hx = V;
+  if (scheme == PERF_SCHEME_COL) hx = ((V + k.den * k.G + V - 1) / V) * V;
+  k.hx = hx;
+  k.row_elems = TW + 2 * hx;
+  // ring: rows a consumer holds for reconstruction + prefetch depth
+  int hold = 1;
+  if (scheme == PERF_SCHEME_ROW) hold = 2;
+  if (scheme == PERF_SCHEME_CHECKER) hold = 2 * k.den - 1;
+  int nr = P->ring > 0 ? next_pow2((int)P->ring) : next_pow2(hold + 10);
+  if (nr < hold + 1) nr = next_pow2(hold + 1);
+  const int nin = P->app == PERF_APP_HOTSPOT ? 2 : 1;
+  const size_t slot_bytes = (size_t)k.row_elems * nin * es;
+  auto bar_bytes = [](int n) { return (size_t)((2 * n * 8 + 127) & ~127); };
+  while (nr > next_pow2(hold + 1) && bar_bytes(nr) + nr * slot_bytes > 200 * 1024) nr >>= 1;
+  k.nr = nr;
+  k.nr_log2 = log2i(nr);
+  smem = bar_bytes(nr) + (size_t)nr * slot_bytes;
+  if (smem > 227 * 1024) return fail(PERF_ERR_UNSUPPORTED, "shared-memory ring exceeds 227 KB");
+  k.seg_h = (int)(P->tile_h > 0 ? P->tile_h : 128);
+  k.n_strips = (P->W + TW - 1) / TW;
+  k.n_segs = (y_end - y_begin + k.seg_h - 1) / k.seg_h;
+  k.frames = frames;
+  const long long g = (long long)k.n_strips * k.n_segs * frames;
+  if (g <= 0 || g > 0x7FFFFFFFLL) return fail(PERF_ERR_INVALID_ARG, "grid size out of range");
+  grid = (unsigned)g;
+  // Rodinia Hotspot coefficients, cell size of the 1024 x 1024 chip (R13)
+  {
+    const double t_chip = 0.0005, chip = 0.016, gw = chip / 1024.0, gh = chip / 1024.0;
+    const double cap = 0.5 * 1.75e6 * t_chip * gw * gh;
+    const double rx = gw / (2.0 * 100.0 * t_chip * gh), ry = gh / (2.0 * 100.0 * t_chip * gw);
+    const double rz = t_chip / (100.0 * gh * gw);
+    const double max_slope = 3.0e6 / (0.5 * t_chip * 1.75e6);
+    const double step = 0.001 / max_slope;
+    k.sdc = (float)(step / cap);
+    k.rx1 = (float)(1.0 / rx);
+    k.ry1 = (float)(1.0 / ry);
+    k.rz1 = (float)(1.0 / rz);
+    k.amb = 80.0f;
+  }
+  return PERF_OK;
+}
+
+static cudaError_t dispatch(const perf_plan_s* P, const KParams& k, unsigned grid, size_t smem, cudaStream_t s) {
+  int scheme = P->rate.num == 0 ? PERF_SCHEME_NONE : P->scheme;
+  const int rc = P->recon;
+  switch (P->app) {
+    case PERF_APP_GAUSSIAN:
+      return P->radius == 1 ? kp::launch_gauss1(scheme, rc, k, grid, smem, s)
+                            : kp::launch_gauss2(scheme, rc, k, grid, smem, s);
+    case PERF_APP_SOBEL:
+      return P->radius == 1 ? kp::launch_sobel1(scheme, rc, k, grid, smem, s)
+                            : kp::launch_sobel2(scheme, rc, k, grid, smem, s);
+    case PERF_APP_MEDIAN: return kp::launch_median(scheme, rc, k, grid, smem, s);
+    case PERF_APP_HOTSPOT: return kp::launch_hotspot(scheme, rc, k, grid, smem, s);
+    case PERF_APP_GAUSS_SOBEL: return kp::launch_gsobel(scheme, rc, k, grid, smem, s);
+    case PERF_APP_INVERSION: return kp::launch_inversion(scheme, rc, k, grid, smem, s);
+  }
+  return cudaErrorInvalidValue;
+}
+
+extern "C" {
+
+const char* perf_last_error(void) { return g_err.c_str(); }
+const char* perf_version(void) { return "kperf 0.1 (sm_100a)"; }
+
+perf_status perf_plan(perf_plan_t* plan, perf_app app, int W, int H, int radius, perf_scheme scheme, perf_rate rate,
+                      perf_recon recon) {
+  if (!plan) return fail(PERF_ERR_INVALID_ARG, "plan is NULL");
+  *plan = nullptr;
+  if (app < PERF_APP_GAUSSIAN || app > PERF_APP_INVERSION) return fail(PERF_ERR_INVALID_ARG, "bad app");
+  if (scheme < PERF_SCHEME_NONE || scheme > PERF_SCHEME_CHECKER) return fail(PERF_ERR_INVALID_ARG, "bad scheme");
+  if (recon != PERF_RECON_NN && recon != PERF_RECON_LINEAR) return fail(PERF_ERR_INVALID_ARG, "bad recon");
+  if (W < 1 || H < 1) return fail(PERF_ERR_INVALID_ARG, "W and H must be >= 1");
+  bool r_ok = false;
+  switch (app) {
+    case PERF_APP_GAUSSIAN:
+    case PERF_APP_SOBEL: r_ok = radius == 1 || radius == 2; break;
+    case PERF_APP_MEDIAN:
+    case PERF_APP_HOTSPOT: r_ok = radius == 1; break;
+    case PERF_APP_GAUSS_SOBEL: r_ok = radius == 2; break;
+    case PERF_APP_INVERSION: r_ok = radius == 0; break;
+  }
+  if (!r_ok) return fail(PERF_ERR_INVALID_ARG, "radius not allowed for this app");
+  if (rate.den < 1 || rate.den > 8) return fail(PERF_ERR_INVALID_ARG, "rate.den must be in [1, 8]");
+  if (!(rate.num == 0 || rate.num == 1 || rate.num == rate.den - 1) || rate.num >= rate.den)
+    return fail(PERF_ERR_INVALID_ARG, "rate.num must be 0, 1 or den-1 (and < den)");
+  if (scheme == PERF_SCHEME_NONE && rate.num != 0)
+    return fail(PERF_ERR_INVALID_ARG, "scheme NONE needs rate.num == 0");
+  if (scheme == PERF_SCHEME_CHECKER && rate.num > 0 && H < rate.den)
+    return fail(PERF_ERR_INVALID_ARG, "checker scheme needs H >= den");
+  perf_plan_s* p = new (std::nothrow) perf_plan_s();
+  if (!p) return fail(PERF_ERR_OOM, "host allocation failed");
+  p->app = app;
+  p->W = W;
+  p->H = H;
+  p->radius = radius;
+  p->scheme = scheme;
+  p->recon = recon;
+  p->rate = rate;
+  p->metric = (app == PERF_APP_SOBEL || app == PERF_APP_GAUSS_SOBEL) ? PERF_METRIC_ME : PERF_METRIC_MRE;
+  *plan = p;
+  return PERF_OK;
+}
+
+perf_status perf_plan_set(perf_plan_t p, int key, long long v) {
+  if (!p) return fail(PERF_ERR_INVALID_ARG, "plan is NULL");
+  switch (key) {
+    case PERF_KEY_BATCH:
+      if (v < 1) return fail(PERF_ERR_INVALID_ARG, "BATCH must be >= 1");
+      p->batch = v;
+      return PERF_OK;
+    case PERF_KEY_ITERS:
+      if (v < 0) return fail(PERF_ERR_INVALID_ARG, "ITERS must be >= 0");
+      p->iters = v;
+      return PERF_OK;
+    case PERF_KEY_GRANULE_BYTES:
+      if (v < (long long)elem_size(p->app) || v % (long long)elem_size(p->app) || v > 4096)
+        return fail(PERF_ERR_INVALID_ARG, "GRANULE_BYTES must be a positive multiple of sizeof(T), <= 4096");
+      p->granule_bytes = v;
+      return PERF_OK;
+    case PERF_KEY_GLOBAL_H:
+      if (v < p->H) return fail(PERF_ERR_INVALID_ARG, "GLOBAL_H must be >= H");
+      p->global_h = v;
+      return PERF_OK;
+    case PERF_KEY_BAND_Y0:
+      if (v < 0) return fail(PERF_ERR_INVALID_ARG, "BAND_Y0 must be >= 0");
+      p->band_y0 = v;
+      return PERF_OK;
+    case PERF_KEY_TILE_W:
+      if (v != kp::kNCW) return fail(PERF_ERR_UNSUPPORTED, "TILE_W: this build provides 4 consumer warps");
+      p->tile_w = v;
+      return PERF_OK;
+    case PERF_KEY_TILE_H:
+      if (v < 1 || v > (1 << 20)) return fail(PERF_ERR_INVALID_ARG, "TILE_H out of range");
+      p->tile_h = v;
+      return PERF_OK;
+    case PERF_KEY_METRIC:
+      if (v < 0 || v > 2) return fail(PERF_ERR_INVALID_ARG, "bad METRIC");
+      p->metric = v;
+      return PERF_OK;
+    case PERF_KEY_LOADER:
+      if (v < 0 || v > 3) return fail(PERF_ERR_INVALID_ARG, "bad LOADER");
+      p->loader = v;
+      return PERF_OK;
+    case PERF_KEY_RING:
+      if (v < 0 || v > 256) return fail(PERF_ERR_INVALID_ARG, "bad RING");
+      p->ring = v;
+      return PERF_OK;
+  }
+  return fail(PERF_ERR_INVALID_ARG, "unknown key");
+}
+
+perf_status perf_plan_get(perf_plan_t p, int key, long long* v) {
+  if (!p || !v) return fail(PERF_ERR_INVALID_ARG, "NULL argument");
+  switch (key) {
+    case PERF_KEY_BATCH: *v = p->batch; return PERF_OK;
+    case PERF_KEY_ITERS: *v = p->iters; return PERF_OK;
+    case PERF_KEY_GRANULE_BYTES: *v = p->granule_bytes; return PERF_OK;
+    case PERF_KEY_GLOBAL_H: *v = p->global_h > 0 ? p->global_h : p->H; return PERF_OK;
+    case PERF_KEY_BAND_Y0: *v = p->band_y0; return PERF_OK;
+    case PERF_KEY_TILE_W: *v = p->tile_w; return PERF_OK;
+    case PERF_KEY_TILE_H: *v = p->tile_h; return PERF_OK;
+    case PERF_KEY_METRIC: *v = p->metric; return PERF_OK;
+    case PERF_KEY_LOADER: *v = p->loader; return PERF_OK;
+    case PERF_KEY_RING: *v = p->ring; return PERF_OK;
+  }
+  return fail(PERF_ERR_INVALID_ARG, "unknown key");
+}
+
+perf_status perf_run(perf_plan_t p, const void* in, void* out, void* stream) {
+  if (!p || !in || !out) return fail(PERF_ERR_INVALID_ARG, "NULL argument");
+  if (p->app == PERF_APP_HOTSPOT) return fail(PERF_ERR_INVALID_ARG, "Hotspot runs through perf_run_hotspot");
+  if (in == out) return fail(PERF_ERR_INVALID_ARG, "in and out must not alias");
+  KParams k;
+  unsigned grid;
+  size_t smem;
+  perf_status st = make_params(p, in, nullptr, out, (int)p->batch, 0, 0, p->H, 0, 0, p->H, k, grid, smem);
+  if (st != PERF_OK) return st;
+  cudaError_t e = dispatch(p, k, grid, smem, static_cast<cudaStream_t>(stream));
+  if (e != cudaSuccess) return cuda_fail(e, "perf_run launch");
+  return PERF_OK;
+}
+
+perf_status perf_run_host(perf_plan_t p, const void* host_in, void* host_out, void* stream) {
+  if (!p || !host_in || !host_out) return fail(PERF_ERR_INVALID_ARG, "NULL argument");
+  if (p->app == PERF_APP_HOTSPOT) return fail(PERF_ERR_UNSUPPORTED, "Hotspot has no host-buffer entry point");
+  const size_t bytes = (size_t)p->batch * p->W * p->H * elem_size(p->app);
+  if (p->stage_bytes < bytes) {
+    if (p->d_stage_in) cudaFree(p->d_stage_in);
+    if (p->d_stage_out) cudaFree(p->d_stage_out);
+    p->d_stage_in = p->d_stage_out = nullptr;
+    p->stage_bytes = 0;
+    if (cudaMalloc(&p->d_stage_in, bytes) != cudaSuccess || cudaMalloc(&p->d_stage_out, bytes) != cudaSuccess)
+      return fail(PERF_ERR_OOM, "staging allocation failed");
+    p->stage_bytes = bytes;
+  }
+  cudaStream_t s = static_cast<cudaStream_t>(stream);
+  CK(cudaMemcpyAsync(p->d_stage_in, host_in, bytes, cudaMemcpyHostToDevice, s));
+  perf_status st = perf_run(p, p->d_stage_in, p->d_stage_out, stream);
+  if (st != PERF_OK) return st;
+  CK(cudaMemcpyAsync(host_out, p->d_stage_out, bytes, cudaMemcpyDeviceToHost, s));
+  CK(cudaStreamSynchronize(s));
+  return PERF_OK;
+}
+
+// ---------------------------------------------------------------- Hotspot ----
+static int band_halo(const perf_plan_s* p) {
+  // stencil radius 1 + distance to the loaded rows a rebuilt row reads
+  const bool vertical = p->rate.num > 0 && (p->scheme == PERF_SCHEME_ROW || p->scheme == PERF_SCHEME_CHECKER);
+  return 1 + (vertical ? p->rate.den : 0);
+}
+
+static perf_status band_alloc(perf_plan_s* p) {
+  const int hb = band_halo(p);
+  const size_t rows = (size_t)p->H + 2 * hb;
+  if (p->band.rows == rows && p->band.hb == hb) return PERF_OK;
+  for (float*& b : p->band.buf) if (b) { cudaFree(b); b = nullptr; }
+  if (p->band.pbuf) { cudaFree(p->band.pbuf); p->band.pbuf = nullptr; }
+  const size_t bytes = rows * p->W * sizeof(float);
+  if (cudaMalloc(&p->band.buf[0], bytes) != cudaSuccess || cudaMalloc(&p->band.buf[1], bytes) != cudaSuccess ||
+      cudaMalloc(&p->band.pbuf, bytes) != cudaSuccess)
+    return fail(PERF_ERR_OOM, "band allocation failed");
+  cudaMemset(p->band.buf[0], 0, bytes);
+  cudaMemset(p->band.buf[1], 0, bytes);
+  cudaMemset(p->band.pbuf, 0, bytes);
+  p->band.rows = rows;
+  p->band.hb = hb;
+  return PERF_OK;
+}
+
+// one step of a band: rows [y0, y0+h) of buffer `src` (with halos filled) -> `dst`
+static perf_status band_step(perf_plan_s* p, const float* src, float* dst, cudaStream_t s) {
+  const int Hg = (int)p->global_h, y0 = (int)p->band_y0, h = p->H, hb = p->band.hb;
+  KParams k;
+  unsigned grid;
+  size_t smem;
+  perf_status st = make_params(p, src, p->band.pbuf, dst, 1, y0 - hb, std::max(0, y0 - hb), std::min(Hg, y0 + h + hb),
+                               y0 - hb, y0, y0 + h, k, grid, smem);
+  if (st != PERF_OK) return st;
+  k.in_fstride = k.out_fstride = 0;
+  cudaError_t e = dispatch(p, k, grid, smem, s);
+  if (e != cudaSuccess) return cuda_fail(e, "hotspot band launch");
+  return PERF_OK;
+}
+
+// NCCL halo exchange of `buf` (rows with halo) between neighbouring bands
+static perf_status band_exchange_nccl(perf_plan_s* p, float* buf, cudaStream_t s) {
+  const int hb = p->band.hb, h = p->H, W = p->W;
+  const size_t n = (size_t)hb * W;
+  if (ncclGroupStart() != ncclSuccess) return fail(PERF_ERR_NCCL, "ncclGroupStart");
+  if (p->rank > 0) {
+    ncclSend(buf + (size_t)hb * W, n, ncclFloat, p->rank - 1, p->comm, s);  // my first rows -> up
+    ncclRecv(buf, n, ncclFloat, p->rank - 1, p->comm, s);                   // its last rows -> my top halo
+  }
+  if (p->rank < p->nranks - 1) {
+    ncclSend(buf + (size_t)h * W, n, ncclFloat, p->rank + 1, p->comm, s);   // my last rows -> down
+    ncclRecv(buf + (size_t)(h + hb) * W, n, ncclFloat, p->rank + 1, p->comm, s);
+  }
+  ncclResult_t r = ncclGroupEnd();
+  if (r != ncclSuccess) return fail(PERF_ERR_NCCL, std::string("halo exchange: ") + ncclGetErrorString(r));
+  return PERF_OK;
+}
+
+perf_status perf_run_hotspot(perf_plan_t p, const float* temp_in, const float* power, float* temp_out, void* stream) {
+  if (!p || !temp_in || !power || !temp_out) return fail(PERF_ERR_INVALID_ARG, "NULL argument");
+  if (p->app != PERF_APP_HOTSPOT) return fail(PERF_ERR_INVALID_ARG, "plan is not a Hotspot plan");
+  if (temp_in == temp_out) return fail(PERF_ERR_INVALID_ARG, "temp_in and temp_out must not alias");
+  cudaStream_t s = static_cast<cudaStream_t>(stream);
+  const long long n = (long long)p->W * p->H;
+  const int Hg = p->global_h > 0 ? (int)p->global_h : p->H;
+  const bool banded = Hg != p->H || p->band_y0 != 0;
+  if (p->iters == 0) {
+    CK(cudaMemcpyAsync(temp_out, temp_in, n * sizeof(float), cudaMemcpyDeviceToDevice, s));
+    return PERF_OK;
+  }
+  if (!banded) {
+    if (p->iters > 1 && p->tmp_elems < (size_t)n) {
+      if (p->d_tmp) cudaFree(p->d_tmp);
+      p->d_tmp = nullptr;
+      if (cudaMalloc(&p->d_tmp, n * sizeof(float)) != cudaSuccess) return fail(PERF_ERR_OOM, "tmp allocation");
+      p->tmp_elems = n;
+    }
+    const float* src = temp_in;
+    for (long long i = 0; i < p->iters; ++i) {
+      float* dst = ((p->iters - 1 - i) % 2 == 0) ? temp_out : p->d_tmp;
+      KParams k;
+      unsigned grid;
+      size_t smem;
+      perf_status st = make_params(p, src, power, dst, 1, 0, 0, p->H, 0, 0, p->H, k, grid, smem);
+      if (st != PERF_OK) return st;
+      cudaError_t e = dispatch(p, k, grid, smem, s);
+      if (e != cudaSuccess) return cuda_fail(e, "hotspot launch");
+      src = dst;
+    }
+    return PERF_OK;
+  }
+  // banded: this rank owns global rows [band_y0, band_y0 + H) of Hg
+  if (!p->comm && p->nranks == 1 && Hg != p->H)
+    return fail(PERF_ERR_INVALID_ARG, "banded Hotspot needs perf_comm_init (or perf_run_hotspot_bands_local)");
+  perf_status st = band_alloc(p);
+  if (st != PERF_OK) return st;
+  const int hb = p->band.hb;
+  if (p->H < hb) return fail(PERF_ERR_UNSUPPORTED, "band thinner than its halo");
+  const size_t W = p->W;
+  CK(cudaMemcpyAsync(p->band.buf[0] + hb * W, temp_in, n * sizeof(float), cudaMemcpyDeviceToDevice, s));
+  CK(cudaMemcpyAsync(p->band.pbuf + hb * W, power, n * sizeof(float), cudaMemcpyDeviceToDevice, s));
+  if ((st = band_exchange_nccl(p, p->band.pbuf, s)) != PERF_OK) return st;
+  int cur = 0;
+  for (long long i = 0; i < p->iters; ++i) {
+    if ((st = band_exchange_nccl(p, p->band.buf[cur], s)) != PERF_OK) return st;
+    if ((st = band_step(p, p->band.buf[cur], p->band.buf[cur ^ 1], s)) != PERF_OK) return st;
+    cur ^= 1;
+  }
+  CK(cudaMemcpyAsync(temp_out, p->band.buf[cur] + hb * W, n * sizeof(float), cudaMemcpyDeviceToDevice, s));
+  return PERF_OK;
+}
+
+/* Single-device emulation of the sharded Hotspot: nb band plans (consecutive
+ * bands of one grid) step in lockstep on `stream`, halos copied device to
+ * device instead of NCCL.  temp_in/power/temp_out are whole-grid buffers. */
+perf_status perf_run_hotspot_bands_local(perf_plan_t* plans, int nb, const float* temp_in, const float* power,
+                                         float* temp_out, void* stream) {
+  if (!plans || nb < 1 || !temp_in || !power || !temp_out) return fail(PERF_ERR_INVALID_ARG, "bad arguments");
+  cudaStream_t s = static_cast<cudaStream_t>(stream);
+  const size_t W = plans[0]->W;
+  const long long iters = plans[0]->iters;
+  for (int b = 0; b < nb; ++b) {
+    perf_plan_s* p = plans[b];
+    if (!p || p->app != PERF_APP_HOTSPOT || (size_t)p->W != W || p->iters != iters)
+      return fail(PERF_ERR_INVALID_ARG, "band plans must be Hotspot plans of one grid");
+    if (b > 0 && p->band_y0 != plans[b - 1]->band_y0 + plans[b - 1]->H)
+      return fail(PERF_ERR_INVALID_ARG, "bands must be consecutive");
+    perf_status st = band_alloc(p);
+    if (st != PERF_OK) return st;
+    if (p->H < p->band.hb) return fail(PERF_ERR_UNSUPPORTED, "band thinner than its halo");
+    const size_t off = (size_t)p->band_y0 * W, n = (size_t)p->H * W, hbw = (size_t)p->band.hb * W;
+    CK(cudaMemcpyAsync(p->band.buf[0] + hbw, temp_in + off, n * sizeof(float), cudaMemcpyDeviceToDevice, s));
+    CK(cudaMemcpyAsync(p->band.pbuf + hbw, power + off, n * sizeof(float), cudaMemcpyDeviceToDevice, s));
+  }
+  auto exchange = [&](int which, bool power_buf) -> perf_status {
+    for (int b = 0; b < nb; ++b) {
+      perf_plan_s* p = plans[b];
+      float* mine = power_buf ? p->band.pbuf : p->band.buf[which];
+      const size_t hb = p->band.hb, h = p->H;
+      if (b > 0) {  // top halo <- last hb rows of band b-1
+        perf_plan_s* q = plans[b - 1];
+        const float* theirs = power_buf ? q->band.pbuf : q->band.buf[which];
+        CK(cudaMemcpyAsync(mine, theirs + (size_t)q->H * W + (q->band.hb - hb) * W, hb * W * sizeof(float),
+                           cudaMemcpyDeviceToDevice, s));
+      }
+      if (b < nb - 1) {  // bottom halo <- first hb rows of band b+1
+        perf_plan_s* q = plans[b + 1];
+        const float* theirs = power_buf ? q->band.pbuf : q->band.buf[which];
+        CK(cudaMemcpyAsync(mine + (hb + h) * W, theirs + (size_t)q->band.hb * W, hb * W * sizeof(float),
+                           cudaMemcpyDeviceToDevice, s));
+      }
+    }
+    return PERF_OK;
+  };
+  perf_status st = exchange(0, true);
+  if (st != PERF_OK) return st;
+  int cur = 0;
+  for (long long i = 0; i < iters; ++i) {
+    if ((st = exchange(cur, false)) != PERF_OK) return st;
+    for (int b = 0; b < nb; ++b)
+      if ((st = band_step(plans[b], plans[b]->band.buf[cur], plans[b]->band.buf[cur ^ 1], s)) != PERF_OK) return st;
+    cur ^= 1;
+  }
+  for (int b = 0; b < nb; ++b) {
+    perf_plan_s* p = plans[b];
+    CK(cudaMemcpyAsync(temp_out + (size_t)p->band_y0 * W, p->band.buf[cur] + (size_t)p->band.hb * W,
+                       (size_t)p->H * W * sizeof(float), cudaMemcpyDeviceToDevice, s));
+  }
+  return PERF_OK;
+}
+
+perf_status perf_error(perf_plan_t p, const void* exact, const void* approx, void* stream, double* err_out,
+                       long long* count_out) {
+  if (!p || !exact || !approx || !err_out) return fail(PERF_ERR_INVALID_ARG, "NULL argument");
+  cudaStream_t s = static_cast<cudaStream_t>(stream);
+  if (!p->d_err) {
+    if (cudaMalloc(&p->d_err, kp::error_scratch_doubles() * sizeof(double)) != cudaSuccess)
+      return fail(PERF_ERR_OOM, "error scratch allocation");
+  }
+  const long long n = (long long)p->batch * p->W * p->H;
+  cudaError_t e = kp::launch_error(p->app == PERF_APP_MEDIAN, exact, approx, n, (int)p->metric, p->d_err, s);
+  if (e != cudaSuccess) return cuda_fail(e, "perf_error launch");
+  double h[3];
+  CK(cudaMemcpyAsync(h, p->d_err + kp::error_scratch_doubles() - 3, sizeof h, cudaMemcpyDeviceToHost, s));
+  CK(cudaStreamSynchronize(s));
+  const long long c = (long long)h[2];
+  if (count_out) *count_out = c;
+  if (p->metric == PERF_METRIC_ME) *err_out = h[1] > 0 ? h[0] / h[1] : 0.0;
+  else *err_out = c > 0 ? h[0] / (double)c : 0.0;
+  return PERF_OK;
+}
+
+perf_status perf_comm_unique_id(void* out) {
+  if (!out) return fail(PERF_ERR_INVALID_ARG, "NULL argument");
+  ncclUniqueId id;
+  ncclResult_t r = ncclGetUniqueId(&id);
+  if (r != ncclSuccess) return fail(PERF_ERR_NCCL, ncclGetErrorString(r));
+  std::memcpy(out, &id, sizeof id);
+  return PERF_OK;
+}
+
+perf_status perf_comm_init(perf_plan_t p, const void* uid, int rank, int nranks) {
+  if (!p || !uid) return fail(PERF_ERR_INVALID_ARG, "NULL argument");
+  if (nranks < 1 || rank < 0 || rank >= nranks) return fail(PERF_ERR_INVALID_ARG, "bad rank / nranks");
+  ncclUniqueId id;
+  std::memcpy(&id, uid, sizeof id);
+  ncclComm_t c;
+  ncclResult_t r = ncclCommInitRank(&c, nranks, id, rank);
+  if (r != ncclSuccess) return fail(PERF_ERR_NCCL, ncclGetErrorString(r));
+  if (p->comm) ncclCommDestroy(p->comm);
+  p->comm = c;
+  p->rank = rank;
+  p->nranks = nranks;
+  return PERF_OK;
+}
+
+perf_status perf_destroy(perf_plan_t p) {
+  if (!p) return PERF_OK;
+  if (p->d_err) cudaFree(p->d_err);
+  if (p->d_tmp) cudaFree(p->d_tmp);
+  if (p->d_stage_in) cudaFree(p->d_stage_in);
+  if (p->d_stage_out) cudaFree(p->d_stage_out);
+  for (float* b : p->band.buf) if (b) cudaFree(b);
+  if (p->band.pbuf) cudaFree(p->band.pbuf);
+  if (p->comm) ncclCommDestroy(p->comm);
+  delete p;
+  return PERF_OK;
+}
+
+}  // extern "C"

@@ -1,0 +1,327 @@
+"""GPU <-> oracle parity through the C ABI.
+
+fp32 apps: |gpu - oracle| <= RTOL*|oracle| + ATOL[app] per element, with
+RTOL = 1e-5 (north_star) and ATOL only for Sobel's cancellation near zero
+(1e-6 x the stencil's magnitude scale sum|w| * 255).  u8 (median): bit-exact.
+Shapes span several CTA tiles (512 fp32 / 2048 u8 columns, 128 rows) and a
+ragged tail; the full BASELINE sizes are checked on sampled pixels.
+"""
+import itertools
+
+import numpy as np
+import pytest
+
+import oracle
+import synth
+
+torch = pytest.importorskip("torch")
+pytestmark = pytest.mark.gpu
+
+import paper_conf_cgo_maiercj18_b200 as kp  # noqa: E402
+
+RTOL = 1e-5
+ATOL = {("gaussian", 1): 0.0, ("gaussian", 2): 0.0, ("inversion", 0): 0.0, ("hotspot", 1): 0.0,
+        ("sobel", 1): 8 * 255e-6, ("sobel", 2): 96 * 255e-6, ("gauss_sobel", 2): 8 * 255e-6}
+
+VARIANTS = [("none", (0, 1), "nn")] + [(s, r, rc) for s in ("row", "col", "checker")
+                                        for r in ((1, 2), (1, 4), (3, 4)) for rc in ("nn", "li")]
+FLOAT_APPS = [("gaussian", 1), ("gaussian", 2), ("sobel", 1), ("sobel", 2), ("inversion", 0),
+              ("gauss_sobel", 2)]
+
+
+@pytest.fixture(scope="module", autouse=True)
+def _cuda():
+    if not torch.cuda.is_available():
+        pytest.skip("no CUDA device")
+    torch.cuda.init()
+
+
+def gpu_run(app, r, img, scheme, rate, recon, G_bytes=32, batch=1, **keys):
+    H, W = img.shape[-2:]
+    dev = torch.from_numpy(np.ascontiguousarray(img)).cuda()
+    out = torch.empty_like(dev)
+    with kp.Plan(app, W, H, r, scheme, rate, recon, granule_bytes=G_bytes, batch=batch, **keys) as p:
+        p.run(dev, out)
+        torch.cuda.synchronize()
+    return out.cpu().numpy()
+
+
+def assert_close(app, r, got, want):
+    if got.dtype == np.uint8:
+        bad = np.argwhere(got != want)
+        assert bad.size == 0, f"{len(bad)} mismatches, first at {bad[:5].tolist()}"
+        return
+    tol = RTOL * np.abs(want) + ATOL[(app, r)]
+    err = np.abs(got.astype(np.float64) - want)
+    bad = np.argwhere(err > tol)
+    assert bad.size == 0, (f"{len(bad)} / {err.size} outside tol; first {bad[:5].tolist()} "
+                           f"got {got[tuple(bad[0])]} want {want[tuple(bad[0])]}")
+
+
+# ---------------------------------------------------------------------------
+@pytest.mark.parametrize("app,r", FLOAT_APPS)
+@pytest.mark.parametrize("scheme,rate,recon", VARIANTS)
+def test_float_apps_parity(app, r, scheme, rate, recon):
+    # 3 strips (last one ragged), 3 segments (last one ragged)
+    W, H = 1100, 300
+    img = synth.image("natural", synth.SEED_C2 + 1, W, H)
+    got = gpu_run(app, r, img, scheme, rate, recon)
+    want = oracle.run(oracle.params(app, W, H, r, scheme, rate, recon, 8), img)
+    assert_close(app, r, got, want)
+
+
+@pytest.mark.parametrize("scheme,rate,recon", VARIANTS)
+def test_median_parity(scheme, rate, recon):
+    W, H = 4200, 140  # 3 strips of 2048 u8 columns, ragged
+    img = synth.image("natural", synth.SEED_C3, W, H, np.uint8)
+    got = gpu_run("median", 1, img, scheme, rate, recon)
+    want = oracle.run(oracle.params("median", W, H, 1, scheme, rate, recon, 32), img)
+    assert_close("median", 1, got, want)
+
+
+@pytest.mark.parametrize("app,r", [("gaussian", 2), ("sobel", 1), ("gauss_sobel", 2), ("median", 1)])
+@pytest.mark.parametrize("shape", [(1, 1), (1, 7), (7, 1), (3, 5), (130, 2), (2, 130), (513, 129), (1027, 33)])
+def test_ragged_and_tiny_shapes(app, r, shape):
+    W, H = shape
+    u8 = app == "median"
+    img = synth.image("pattern", 17, W, H, np.uint8 if u8 else np.float32)
+    G = 32 if u8 else 8
+    for scheme, rate, recon in [("none", (0, 1), "nn"), ("row", (1, 2), "li"), ("col", (1, 4), "nn"),
+                                ("checker", (1, 2), "li"), ("row", (3, 4), "nn")]:
+        if scheme == "checker" and H < rate[1]:
+            continue
+        got = gpu_run(app, r, img, scheme, rate, recon)
+        want = oracle.run(oracle.params(app, W, H, r, scheme, rate, recon, G), img)
+        assert_close(app, r, got, want)
+
+
+@pytest.mark.parametrize("gbytes", [4, 12, 16, 64, 128])
+def test_granule_sizes(gbytes):
+    """G not a multiple of the lane chunk (4 fp32) takes the generic rebuild path."""
+    W, H = 1024, 64
+    img = synth.image("natural", 5, W, H)
+    for scheme, rate, recon in [("col", (1, 2), "li"), ("checker", (3, 4), "nn"), ("col", (7, 8), "li")]:
+        got = gpu_run("gaussian", 2, img, scheme, rate, recon, G_bytes=gbytes)
+        want = oracle.run(oracle.params("gaussian", W, H, 2, scheme, rate, recon, gbytes // 4), img)
+        assert_close("gaussian", 2, got, want)
+
+
+@pytest.mark.parametrize("den", [2, 3, 5, 6, 7, 8])
+def test_all_denominators(den):
+    W, H = 600, 90
+    img = synth.image("natural", 31, W, H)
+    for scheme in ("row", "col", "checker"):
+        for num in sorted({1, den - 1}):
+            for recon in ("nn", "li"):
+                got = gpu_run("sobel", 1, img, scheme, (num, den), recon)
+                want = oracle.run(oracle.params("sobel", W, H, 1, scheme, (num, den), recon, 8), img)
+                assert_close("sobel", 1, got, want)
+
+
+# ---------------------------------------------------------------------------
+# invariants of the CUDA path itself
+def test_rate0_bit_identical_to_exact():
+    W, H = 1030, 200
+    img = synth.image("natural", 3, W, H)
+    ex = gpu_run("gaussian", 2, img, "none", (0, 1), "nn")
+    for s in ("row", "col", "checker"):
+        assert np.array_equal(gpu_run("gaussian", 2, img, s, (0, 4), "li"), ex)
+
+
+def test_loaders_and_tiles_give_identical_bits():
+    W, H = 2048, 260
+    img = synth.image("natural", 9, W, H)
+    for scheme, rate, recon, loaders in [("row", (1, 2), "li", (1, 2, 3)), ("none", (0, 1), "nn", (1, 2, 3)),
+                                         ("col", (1, 4), "nn", (2, 3)), ("checker", (3, 4), "li", (2, 3))]:
+        ref = gpu_run("sobel", 2, img, scheme, rate, recon)
+        for ld in loaders:
+            for th in (1, 7, 128, 1000):
+                got = gpu_run("sobel", 2, img, scheme, rate, recon, loader=ld, tile_h=th)
+                assert np.array_equal(got, ref), (scheme, ld, th)
+
+
+def test_constant_image_rebuilds_exactly():
+    W, H = 700, 150
+    img = np.full((H, W), 93.0, dtype=np.float32)
+    for s, rate, rc in VARIANTS:
+        assert np.all(gpu_run("gaussian", 2, img, s, rate, rc) == 93.0)
+        assert np.all(gpu_run("sobel", 1, img, s, rate, rc) == 0.0)
+
+
+def test_batch_frames():
+    W, H, B = 520, 70, 3
+    imgs = np.stack([synth.image("natural", 100 + b, W, H) for b in range(B)])
+    got = gpu_run("gaussian", 2, imgs, "row", (1, 2), "li", batch=B)
+    for b in range(B):
+        want = oracle.run(oracle.params("gaussian", W, H, 2, "row", (1, 2), "li"), imgs[b])
+        assert_close("gaussian", 2, got[b], want)
+
+
+def test_run_host_equals_run():
+    W, H = 640, 96
+    img = synth.image("natural", 4, W, H)
+    out = np.zeros_like(img)
+    with kp.Plan("sobel", W, H, 1, "checker", (1, 2), "li") as p:
+        p.run_host(img, out)
+    assert np.array_equal(out, gpu_run("sobel", 1, img, "checker", (1, 2), "li"))
+
+
+def test_device_generator_matches_host():
+    for cls in ("flat", "natural", "pattern"):
+        d = torch.empty((2, 300, 500), dtype=torch.float32, device="cuda")
+        synth.image_device(cls, 77, 500, 300, 2, d.data_ptr(), False)
+        u = torch.empty((300, 500), dtype=torch.uint8, device="cuda")
+        synth.image_device(cls, 77, 500, 300, 1, u.data_ptr(), True)
+        torch.cuda.synchronize()
+        assert np.array_equal(d[0].cpu().numpy(), synth.image(cls, 77, 500, 300))
+        assert np.array_equal(d[1].cpu().numpy(), synth.image(cls, 78, 500, 300))
+        assert np.array_equal(u.cpu().numpy(), synth.image(cls, 77, 500, 300, np.uint8))
+    T = torch.empty((64, 96), device="cuda")
+    P = torch.empty((64, 96), device="cuda")
+    synth.hotspot_device(5, 96, 64, T.data_ptr(), P.data_ptr())
+    torch.cuda.synchronize()
+    Th, Ph = synth.hotspot(5, 96, 64)
+    assert np.array_equal(T.cpu().numpy(), Th) and np.array_equal(P.cpu().numpy(), Ph)
+
+
+# ---------------------------------------------------------------------------
+# error metric (a5)
+@pytest.mark.parametrize("app,r,metric", [("gaussian", 2, "mre"), ("sobel", 1, "me"), ("median", 1, "mre"),
+                                          ("gaussian", 2, "mae")])
+def test_error_metric(app, r, metric):
+    W, H = 1500, 333
+    u8 = app == "median"
+    img = synth.image("natural", 12, W, H, np.uint8 if u8 else np.float32)
+    ex = gpu_run(app, r, img, "none", (0, 1), "nn")
+    ap = gpu_run(app, r, img, "row", (1, 2), "li")
+    with kp.Plan(app, W, H, r, "row", (1, 2), "li", metric=kp.METRIC[metric]) as p:
+        v, c = p.error(torch.from_numpy(ex).cuda(), torch.from_numpy(ap).cuda())
+    # same buffers through the oracle's metric
+    ov, oc = oracle.error(metric, ex, ap)
+    assert c == oc
+    assert abs(v - ov) <= 1e-9 * max(1.0, abs(ov))
+    # end to end: the oracle's own exact/perforated outputs (north_star: 1e-6)
+    oe = oracle.run(oracle.params(app, W, H, r, "none", (0, 1), "nn", 32 if u8 else 8), img)
+    oa = oracle.run(oracle.params(app, W, H, r, "row", (1, 2), "li", 32 if u8 else 8), img)
+    assert abs(v - oracle.error(metric, oe, oa)[0]) <= 1e-6
+
+
+# ---------------------------------------------------------------------------
+# Hotspot (a6)
+@pytest.mark.parametrize("scheme,rate,recon", [("none", (0, 1), "nn"), ("row", (1, 2), "nn"),
+                                               ("row", (1, 2), "li"), ("row", (3, 4), "li"),
+                                               ("col", (1, 2), "li"), ("checker", (1, 4), "nn")])
+@pytest.mark.parametrize("iters", [1, 6])
+def test_hotspot_parity(scheme, rate, recon, iters):
+    W, H = 1100, 260
+    T, P = synth.hotspot(synth.SEED_C4, W, H)
+    Td, Pd = torch.from_numpy(T).cuda(), torch.from_numpy(P).cuda()
+    out = torch.empty_like(Td)
+    with kp.Plan("hotspot", W, H, 1, scheme, rate, recon, iters=iters) as p:
+        p.hotspot(Td, Pd, out)
+        torch.cuda.synchronize()
+    want = oracle.hotspot(oracle.params("hotspot", W, H, 1, scheme, rate, recon, 8), T, P, iters)
+    assert_close("hotspot", 1, out.cpu().numpy(), want)
+    assert np.array_equal(Td.cpu().numpy(), T)  # temp_in untouched
+
+
+@pytest.mark.parametrize("scheme,rate,recon", [("none", (0, 1), "nn"), ("row", (1, 2), "li"),
+                                               ("row", (3, 4), "nn"), ("checker", (1, 2), "li")])
+@pytest.mark.parametrize("nb", [2, 3, 4])
+def test_hotspot_bands_equal_whole_grid(scheme, rate, recon, nb):
+    """Sharding semantics: row bands with halo exchange == one grid, bit for bit."""
+    W, H, iters = 640, 200, 9
+    T, P = synth.hotspot(7, W, H)
+    Td, Pd = torch.from_numpy(T).cuda(), torch.from_numpy(P).cuda()
+    whole = torch.empty_like(Td)
+    with kp.Plan("hotspot", W, H, 1, scheme, rate, recon, iters=iters) as p:
+        p.hotspot(Td, Pd, whole)
+    cuts = np.linspace(0, H, nb + 1).astype(int)
+    cuts[1:-1] += 3  # uneven bands
+    plans = []
+    for b in range(nb):
+        h = int(cuts[b + 1] - cuts[b])
+        plans.append(kp.Plan("hotspot", W, h, 1, scheme, rate, recon, iters=iters, global_h=H,
+                             band_y0=int(cuts[b])))
+    banded = torch.empty_like(Td)
+    kp.perf_run_hotspot_bands_local([q.handle for q in plans], Td, Pd, banded)
+    torch.cuda.synchronize()
+    assert torch.equal(banded, whole)
+    for q in plans:
+        q.close()
+
+
+# ---------------------------------------------------------------------------
+# BASELINE sizes in the bench's launch configuration, sampled pixels
+def _samples(W, H, n, seed):
+    rng = np.random.default_rng(seed)
+    xs = np.r_[0, W - 1, 0, W - 1, rng.integers(0, W, n)]
+    ys = np.r_[0, 0, H - 1, H - 1, rng.integers(0, H, n)]
+    return xs, ys
+
+
+def test_c1_full_image():
+    W = H = 512
+    img = synth.image("natural", synth.SEED_C1, W, H)
+    got = gpu_run("gaussian", 2, img, "row", (1, 2), "li")
+    want = oracle.run(oracle.params("gaussian", W, H, 2, "row", (1, 2), "li"), img)
+    assert_close("gaussian", 2, got, want)
+
+
+@pytest.mark.parametrize("app,r", [("gaussian", 2), ("sobel", 1)])
+@pytest.mark.parametrize("scheme,rate,recon", [(s, r, rc) for s in ("row", "col", "checker")
+                                               for r in ((1, 2), (1, 4)) for rc in ("nn", "li")])
+def test_c2_sampled(app, r, scheme, rate, recon):
+    W = H = 4096
+    img = synth.image("natural", synth.SEED_C2 + 1, W, H)
+    got = gpu_run(app, r, img, scheme, rate, recon)
+    xs, ys = _samples(W, H, 400, 2)
+    want = oracle.run_pixels(oracle.params(app, W, H, r, scheme, rate, recon, 8), img, xs, ys)
+    assert_close(app, r, got[ys, xs], want)
+
+
+def test_c3_sampled():
+    W = H = 8192
+    img = synth.image("natural", synth.SEED_C3, W, H, np.uint8)
+    for rate in ((1, 2), (1, 4), (3, 4)):
+        got = gpu_run("median", 1, img, "col", rate, "nn")
+        xs, ys = _samples(W, H, 2000, 3)
+        want = oracle.run_pixels(oracle.params("median", W, H, 1, "col", rate, "nn", 32), img, xs, ys)
+        assert np.array_equal(got[ys, xs], want)
+
+
+def test_c4_hotspot_cone_sampled():
+    """4096^2 x 40 steps; oracle on the dependency cones of a few patches."""
+    W = H = 4096
+    iters = 40
+    T = torch.empty((H, W), device="cuda")
+    P = torch.empty((H, W), device="cuda")
+    synth.hotspot_device(synth.SEED_C4, W, H, T.data_ptr(), P.data_ptr())
+    out = torch.empty_like(T)
+    with kp.Plan("hotspot", W, H, 1, "row", (1, 2), "li", iters=iters) as p:
+        p.hotspot(T, P, out)
+    torch.cuda.synchronize()
+    Th, Ph = T.cpu().numpy(), P.cpu().numpy()
+    o = out.cpu().numpy()
+    prm = oracle.params("hotspot", W, H, 1, "row", (1, 2), "li")
+    for x0, y0 in [(0, 0), (2000, 1500), (4090, 4090), (777, 4093)]:
+        w = min(6, W - x0)
+        h = min(3, H - y0)
+        want = oracle.hotspot_rect(prm, Th, Ph, iters, x0, y0, w, h)
+        assert_close("hotspot", 1, o[y0:y0 + h, x0:x0 + w], want)
+
+
+def test_c5_frames_sampled():
+    W, H, B = 3840, 2160, 4
+    frames = torch.empty((B, H, W), device="cuda")
+    synth.image_device("natural", synth.SEED_C5, W, H, B, frames.data_ptr(), False)
+    out = torch.empty_like(frames)
+    with kp.Plan("gauss_sobel", W, H, 2, "row", (1, 2), "li", batch=B) as p:
+        p.run(frames, out)
+    torch.cuda.synchronize()
+    prm = oracle.params("gauss_sobel", W, H, 2, "row", (1, 2), "li")
+    for b in (0, B - 1):
+        img = synth.image("natural", synth.SEED_C5 + b, W, H)
+        xs, ys = _samples(W, H, 300, 10 + b)
+        want = oracle.run_pixels(prm, img, xs, ys)
+        assert_close("gauss_sobel", 2, out[b].cpu().numpy()[ys, xs], want)
