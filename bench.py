@@ -196,7 +196,7 @@ def oracle_sample(cfg, rows=256):
         return (n * rows) / (time.perf_counter() - t0), f"1 Hotspot step on a {n}x{rows} grid"
     u8 = app == "median"
     img = synth.image(cfg["cls"], cfg["seed"], W, rows, np.uint8 if u8 else np.float32)
-    prm = oracle.params(app, W, rows, cfg["r"], cfg["scheme"], cfg["rate"], cfg["recon"], 32 if u8 else 8)
+    prm = oracle.params(app, W, rows, cfg["r"], cfg["scheme"], cfg["rate"], cfg["recon"], 128 if u8 else 32)
     t0 = time.perf_counter()
     oracle.run(prm, img)
     return (W * rows) / (time.perf_counter() - t0), f"{W}x{rows} rows of one frame"
@@ -290,7 +290,7 @@ def main():
         synth.image_device(cfg["cls"], cfg["seed"] + rank * B, W, H, B, x.data_ptr(), u8, stream.cuda_stream)
         y = torch.empty_like(x)
         yex = torch.empty_like(x)
-        G = 32 if u8 else 32
+        G = 128  # the measured B200 DRAM fill granule (tools/granule_probe.cu)
         plan = kp.Plan(app, W, H, cfg["r"], cfg["scheme"], cfg["rate"], cfg["recon"], batch=B, granule_bytes=G)
         exact = kp.Plan(app, W, H, cfg["r"], "none", (0, 1), "nn", batch=B)
         run = lambda: plan.run(x, y, stream)  # noqa: E731

@@ -86,7 +86,8 @@ typedef struct perf_plan_s* perf_plan_t;
 enum {
   PERF_KEY_BATCH = 1,          /* frames per perf_run (default 1) */
   PERF_KEY_ITERS = 2,          /* Hotspot steps per perf_run_hotspot (default 1) */
-  PERF_KEY_GRANULE_BYTES = 3,  /* G * sizeof(T) for COL/CHECKER (default 32; multiple of sizeof(T)) */
+  PERF_KEY_GRANULE_BYTES = 3,  /* G * sizeof(T) for COL/CHECKER (default 128 = the measured B200 DRAM
+                                  fill granule; smaller cells save no DRAM bytes; multiple of sizeof(T)) */
   PERF_KEY_GLOBAL_H = 4,       /* sharded Hotspot: rows of the whole grid (default H) */
   PERF_KEY_BAND_Y0 = 5,        /* sharded Hotspot: first global row of this rank's band (default 0) */
   PERF_KEY_TILE_W = 6,         /* consumer warps per CTA (1..8); tile width = warps * 32 * V */

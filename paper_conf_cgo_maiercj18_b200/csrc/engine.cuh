@@ -42,6 +42,7 @@ struct KParams {
   int num, den, G, keep_one; // skipped fraction num/den, granule G (pixels)
   int loader;
   int seg_h, n_strips, n_segs, frames;
+  int seg_auto;              // seg_h is an upper bound; the launcher picks the wave-filling value
   int nr, nr_log2;           // ring slots (power of two)
   int hx;                    // columns of halo/apron each side (multiple of V)
   int row_elems;             // TW + 2*hx
@@ -193,11 +194,12 @@ __device__ __forceinline__ int row_of_idx(const Mask& m, const RowPlan& rp, int 
 
 // ---------------------------------------------------------------------------
 // producer warp: fetch the kept part of every needed row into the ring
-template <typename T, int SCHEME, int NIN, int NCW>
+// g0: global (per-CTA, across work items) index of this item's first load;
+// ring slot = g & (nr-1), fill phase = g >> log2(nr).
+template <typename T, int SCHEME, int NIN, int TW>
 __device__ __forceinline__ void producer(const KParams& p, const Mask& m, const RowPlan& rp, int x0, int frame,
-                                         uint64_t* full, uint64_t* empty, T* ring) {
-  constexpr int V = VT<T>::V;
-  constexpr int TW = NCW * 32 * V;
+                                         int g0, uint64_t* full, uint64_t* empty, T* ring) {
+  constexpr int V = VT<T>::V;  // 16-B load chunk
   const int lane = threadIdx.x & 31;
   const int cx0 = max(x0 - p.hx, 0);
   const int cx1 = min(x0 + TW + p.hx, p.W);
@@ -217,8 +219,9 @@ __device__ __forceinline__ void producer(const KParams& p, const Mask& m, const 
   }
 
   for (int i = 0; i < rp.nload; ++i) {
-    const int slot = i & (p.nr - 1);
-    if (i >= p.nr) mbar_wait(&empty[slot], ((i >> p.nr_log2) - 1) & 1);
+    const int g = g0 + i;
+    const int slot = g & (p.nr - 1);
+    if (g >= p.nr) mbar_wait(&empty[slot], ((g >> p.nr_log2) - 1) & 1);
     const int y = row_of_idx<SCHEME>(m, rp, i);
     const long long roff = (long long)(y - p.in_row0) * p.W;
     T* dst = ring + slot * slot_elems;
@@ -269,31 +272,225 @@ __device__ __forceinline__ void producer(const KParams& p, const Mask& m, const 
   }
 }
 
+
 // ---------------------------------------------------------------------------
-// consumer-side rebuild of one lane chunk (V samples starting at column xc)
-struct RowCtx {
-  int y, ym;
-  int kept;                // row scheme: this row loaded
-  int slot_c;              // ring slot of row y (row scheme: if kept; others: always)
-  int slot_a, slot_b;      // row scheme: slots of the loaded rows below/above
-  int has_a, has_b, da, db;
+// consumer side: fragments of N consecutive samples held in registers
+template <typename T, int N>
+struct Frag;
+
+template <int N>
+struct Frag<float, N> {
+  float v[N];
+  __device__ __forceinline__ float get(int i) const { return v[i]; }
+  __device__ __forceinline__ void set(int i, float s) { v[i] = s; }
+  __device__ __forceinline__ static Frag splat(float s) {
+    Frag f;
+#pragma unroll
+    for (int i = 0; i < N; ++i) f.v[i] = s;
+    return f;
+  }
 };
 
-struct ChunkInfo {  // per-lane, row-independent facts of a chunk
+template <int N>
+struct Frag<uint8_t, N> {  // N bytes packed little-endian in N/4 words
+  uint32_t w[N / 4];
+  __device__ __forceinline__ uint8_t get(int i) const { return (uint8_t)(w[i >> 2] >> (8 * (i & 3))); }
+  __device__ __forceinline__ void set(int i, uint8_t s) {
+    const int k = i >> 2, sh = 8 * (i & 3);
+    w[k] = (w[k] & ~(0xFFu << sh)) | ((uint32_t)s << sh);
+  }
+  __device__ __forceinline__ static Frag splat(uint8_t s) {
+    Frag f;
+#pragma unroll
+    for (int k = 0; k < N / 4; ++k) f.w[k] = 0x01010101u * s;
+    return f;
+  }
+};
+
+template <typename T, int N>
+__device__ __forceinline__ Frag<T, N> ldf(const T* p) {
+  Frag<T, N> f;
+  constexpr int B = N * (int)sizeof(T);
+  static_assert(B == 4 || B == 8 || B == 16 || B == 32, "fragment size");
+  if constexpr (B == 32) {
+    reinterpret_cast<uint4*>(&f)[0] = reinterpret_cast<const uint4*>(p)[0];
+    reinterpret_cast<uint4*>(&f)[1] = reinterpret_cast<const uint4*>(p)[1];
+  } else if constexpr (B == 16) *reinterpret_cast<uint4*>(&f) = *reinterpret_cast<const uint4*>(p);
+  else if constexpr (B == 8) *reinterpret_cast<uint2*>(&f) = *reinterpret_cast<const uint2*>(p);
+  else *reinterpret_cast<uint32_t*>(&f) = *reinterpret_cast<const uint32_t*>(p);
+  return f;
+}
+
+// LI of two loaded fragments with a common span: (a*db + b*da) / (da + db)
+template <int N>
+__device__ __forceinline__ Frag<float, N> li_frag(const Frag<float, N>& a, const Frag<float, N>& b, int da,
+                                                  int db) {
+  Frag<float, N> r;
+  if (da == db) {
+#pragma unroll
+    for (int i = 0; i < N; ++i) r.v[i] = __fmul_rn(__fadd_rn(a.v[i], b.v[i]), 0.5f);
+  } else {
+    const float fda = (float)da, fdb = (float)db, inv = __frcp_rn((float)(da + db));
+#pragma unroll
+    for (int i = 0; i < N; ++i) r.v[i] = VT<float>::li(a.v[i], b.v[i], fda, fdb, inv);
+  }
+  return r;
+}
+
+template <int N>
+__device__ __forceinline__ Frag<uint8_t, N> li_frag(const Frag<uint8_t, N>& a, const Frag<uint8_t, N>& b,
+                                                    int da, int db) {
+  Frag<uint8_t, N> r;
+  if (da == db) {  // (a + b + 1) >> 1 per byte
+#pragma unroll
+    for (int k = 0; k < N / 4; ++k) r.w[k] = (a.w[k] | b.w[k]) - (((a.w[k] ^ b.w[k]) >> 1) & 0x7F7F7F7Fu);
+  } else {
+    const uint32_t mg = VT<uint8_t>::magic_of(da + db);
+#pragma unroll
+    for (int i = 0; i < N; ++i) r.set(i, (uint8_t)VT<uint8_t>::li_int(a.get(i), b.get(i), da, db, mg));
+  }
+  return r;
+}
+
+__device__ __forceinline__ float li_px(float a, float b, int da, int db) { return VT<float>::li1(a, b, da, db); }
+__device__ __forceinline__ uint8_t li_px(uint8_t a, uint8_t b, int da, int db) {
+  return VT<uint8_t>::li1(a, b, da, db);
+}
+
+// A row recipe: everything a consumer needs to rebuild one virtual input row,
+// computed once per CTA into shared memory.
+//   y     clamped global row;  need = need_hi | need_lo << 16 (ring indices)
+//   info  slot_a | slot_b << 8 | ym << 16 | da << 20 | db << 24 | kept << 28 |
+//         li << 29 | has_a << 30 | has_b << 31
+//   wa    LI weight of the lower sample: value = b + (a - b) * wa, wa = db/(da+db)
+// Row scheme: a kept row, and an NN-rebuilt row, are plain copies of slot_a.
+struct Recipe {
+  int y, need;
+  uint32_t info;
+  float wa;
+};
+
+__device__ __forceinline__ int rc_slot_a(uint32_t i) { return (int)(i & 0xFF); }
+__device__ __forceinline__ int rc_slot_b(uint32_t i) { return (int)((i >> 8) & 0xFF); }
+__device__ __forceinline__ int rc_ym(uint32_t i) { return (int)((i >> 16) & 0xF); }
+__device__ __forceinline__ int rc_da(uint32_t i) { return (int)((i >> 20) & 0xF); }
+__device__ __forceinline__ int rc_db(uint32_t i) { return (int)((i >> 24) & 0xF); }
+__device__ __forceinline__ bool rc_kept(uint32_t i) { return (i >> 28) & 1; }
+__device__ __forceinline__ bool rc_li(uint32_t i) { return (i >> 29) & 1; }
+__device__ __forceinline__ bool rc_has_a(uint32_t i) { return (i >> 30) & 1; }
+__device__ __forceinline__ bool rc_has_b(uint32_t i) { return (i >> 31) & 1; }
+
+template <int SCHEME, int RECON>
+__device__ __forceinline__ Recipe make_recipe(const KParams& p, const Mask& m, const RowPlan& rp, int vy) {
+  Recipe r;
+  const int y = clampi(vy, rp.lim_lo, rp.lim_hi);
+  const int ym = y % m.den, nmask = p.nr - 1;
+  int need_hi, need_lo, sa = 0, sb = 0, da = 1, db = 1, kept = 1, li = 0, ha = 0, hb = 0;
+  float wa = 1.f;
+  if (SCHEME == S_ROW) {
+    kept = m.phase_kept(ym);
+    if (kept) {
+      const int id = m.ord(y) - rp.ord_lo;
+      sa = sb = id & nmask;
+      need_hi = need_lo = id;
+    } else {
+      da = m.dlo(ym);
+      db = m.dhi(ym);
+      ha = (y - da) >= rp.lo;
+      hb = (y + db) <= rp.hi;
+      const int ida = m.ord(y - da) - rp.ord_lo;
+      const int idb = hb ? m.ord(y + db) - rp.ord_lo : ida;
+      need_hi = hb ? idb : ida;
+      need_lo = ha ? ida : idb;
+      if (RECON == R_LI && ha && hb) {
+        li = 1;
+        sa = ida & nmask;
+        sb = idb & nmask;
+        wa = __fdiv_rn((float)db, (float)(da + db));
+      } else {  // nearest neighbour: a copy of the chosen loaded row
+        kept = 1;
+        sa = sb = ((!hb || (ha && da <= db)) ? ida : idb) & nmask;
+      }
+    }
+  } else if (SCHEME == S_CHECKER) {
+    sa = sb = (y - rp.lo) & nmask;
+    need_hi = min(y + m.den - 1, rp.hi) - rp.lo;
+    need_lo = max(y - (m.den - 1), rp.lo) - rp.lo;
+  } else {
+    sa = sb = (y - rp.lo) & nmask;
+    need_hi = need_lo = y - rp.lo;
+  }
+  r.y = y;
+  r.need = need_hi | (need_lo << 16);
+  r.info = (uint32_t)sa | ((uint32_t)sb << 8) | ((uint32_t)ym << 16) | ((uint32_t)da << 20) |
+           ((uint32_t)db << 24) | ((uint32_t)kept << 28) | ((uint32_t)li << 29) | ((uint32_t)ha << 30) |
+           ((uint32_t)hb << 31);
+  r.wa = wa;
+  return r;
+}
+
+// b + (a - b) * wa, elementwise
+template <int N>
+__device__ __forceinline__ Frag<float, N> lerp_frag(const Frag<float, N>& a, const Frag<float, N>& b, float wa) {
+  Frag<float, N> r;
+  if constexpr (N % 2 == 0) {  // paired fp32: FADD2 + FFMA2 per two samples
+    const f2 w = splat2(wa);
+#pragma unroll
+    for (int i = 0; i < N; i += 2) {
+      const f2 bb = pk2(b.v[i], b.v[i + 1]);
+      up2(fma2(sub2(pk2(a.v[i], a.v[i + 1]), bb), w, bb), r.v[i], r.v[i + 1]);
+    }
+  } else {
+#pragma unroll
+    for (int i = 0; i < N; ++i) r.v[i] = fmaf(a.v[i] - b.v[i], wa, b.v[i]);
+  }
+  return r;
+}
+
+struct RowCtx {
+  int y, ym;
+  int kept;           // row scheme: row y loaded
+  int slot_c;         // ring slot of row y (row scheme: when kept)
+  int slot_a, slot_b; // row scheme: slots of the loaded rows below/above
+  int has_a, has_b, da, db;
+  float wa;           // row scheme LI weight (see Recipe)
+};
+
+// generic-path context from a recipe
+template <int SCHEME>
+__device__ __forceinline__ RowCtx ctx_of(const Recipe& r) {
+  RowCtx c;
+  c.y = r.y;
+  c.ym = rc_ym(r.info);
+  c.kept = SCHEME == S_ROW ? (rc_kept(r.info) ? 1 : 0) : 1;
+  c.slot_c = rc_slot_a(r.info);
+  c.slot_a = rc_slot_a(r.info);
+  c.slot_b = rc_slot_b(r.info);
+  c.has_a = rc_has_a(r.info);
+  c.has_b = rc_has_b(r.info);
+  c.da = rc_da(r.info);
+  c.db = rc_db(r.info);
+  c.wa = r.wa;
+  return c;
+}
+
+struct ChunkInfo {  // per-lane, row-independent facts of a V-aligned chunk
   int xc;           // first global column
-  int fast;         // inside the image and mask-uniform
   int gxm;          // (xc / G) % den
-  int col_kept, xa, xb;  // column scheme: kept?, nearest loaded columns (or -1)
+  int col_kept, xa, xb;  // column scheme: loaded?, nearest loaded columns below/above (xb = -1: none)
 };
 
 template <int SCHEME>
-__device__ __forceinline__ ChunkInfo make_chunk(const KParams& p, const Mask& m, int xc, int V) {
+__device__ __forceinline__ ChunkInfo make_chunk(const KParams& p, const Mask& m, int xc) {
   ChunkInfo c;
   c.xc = xc;
-  c.fast = p.fast_ok && xc >= 0 && xc + V <= p.W;
-  c.gxm = 0; c.col_kept = 1; c.xa = -1; c.xb = -1;
-  if ((SCHEME == S_COL || SCHEME == S_CHECKER) && xc >= 0) c.gxm = (xc / p.G) % m.den;
-  if (SCHEME == S_COL && xc >= 0) {
+  c.gxm = 0;
+  c.col_kept = 1;
+  c.xa = 0;
+  c.xb = -1;
+  if (xc < 0 || xc >= p.W) return c;  // outside: treated as loaded (value replaced by the clamp)
+  if (SCHEME == S_COL || SCHEME == S_CHECKER) c.gxm = (xc / p.G) % m.den;
+  if (SCHEME == S_COL) {
     const int gx = xc / p.G, t = c.gxm;
     c.col_kept = m.phase_kept(t);
     if (!c.col_kept) {
@@ -305,35 +502,99 @@ __device__ __forceinline__ ChunkInfo make_chunk(const KParams& p, const Mask& m,
   return c;
 }
 
+// fast rebuild of N samples at ring column `col` (global column fx), all in one
+// mask cell described by `ci`; row facts from the recipe
+template <typename T, int N, int SCHEME, int RECON>
+__device__ __forceinline__ Frag<T, N> rebuild_frag(const KParams& p, const Mask& m, const RowPlan& rp,
+                                                   const Recipe& rec, const ChunkInfo& ci, const T* ring,
+                                                   int slot_elems, int col, int fx, int base) {
+  const uint32_t info = rec.info;
+  if (SCHEME == S_NONE) return ldf<T, N>(ring + rc_slot_a(info) * slot_elems + col);
+  if (SCHEME == S_ROW) {
+    if (RECON == R_NN || rc_kept(info)) return ldf<T, N>(ring + rc_slot_a(info) * slot_elems + col);
+    const Frag<T, N> a = ldf<T, N>(ring + rc_slot_a(info) * slot_elems + col);
+    const Frag<T, N> b = ldf<T, N>(ring + rc_slot_b(info) * slot_elems + col);
+    if constexpr (sizeof(T) == 4) return lerp_frag<N>(a, b, rec.wa);
+    else return li_frag<N>(a, b, rc_da(info), rc_db(info));
+  }
+  RowCtx rc;
+  rc.y = rec.y;
+  rc.ym = rc_ym(info);
+  rc.slot_c = rc_slot_a(info);
+  if (SCHEME == S_CHECKER) {
+    int t = ci.gxm + rc.ym;
+    if (t >= m.den) t -= m.den;
+    if (m.phase_kept(t)) return ldf<T, N>(ring + rc.slot_c * slot_elems + col);
+    const int da = m.dlo(t), db = m.dhi(t);
+    const int ya = rc.y - da, yb = rc.y + db;
+    const bool ha = ya >= rp.lim_lo, hb = yb <= rp.lim_hi;
+    const int sa = (ya - rp.lo) & (p.nr - 1), sb = (yb - rp.lo) & (p.nr - 1);
+    if (RECON == R_LI && ha && hb)
+      return li_frag<N>(ldf<T, N>(ring + sa * slot_elems + col), ldf<T, N>(ring + sb * slot_elems + col), da, db);
+    const int s = (!hb || (ha && da <= db)) ? sa : sb;
+    return ldf<T, N>(ring + s * slot_elems + col);
+  }
+  // column scheme: rebuilt along x from the edge samples of the nearest loaded granules
+  const T* row = ring + rc.slot_c * slot_elems;
+  if (ci.col_kept) return ldf<T, N>(row + col);
+  const T a = row[ci.xa - base];
+  const bool hb = ci.xb >= 0;
+  const T b = hb ? row[ci.xb - base] : a;
+  Frag<T, N> r;
+  if (RECON == R_LI && hb) {
+    if constexpr (sizeof(T) == 4) {
+      const float inv = __frcp_rn((float)(ci.xb - ci.xa));
+#pragma unroll
+      for (int i = 0; i < N; ++i) {
+        const int da = fx + i - ci.xa, db = ci.xb - fx - i;
+        r.set(i, VT<float>::li(a, b, (float)da, (float)db, inv));
+      }
+    } else {
+      const uint32_t mg = VT<uint8_t>::magic_of(ci.xb - ci.xa);
+#pragma unroll
+      for (int i = 0; i < N; ++i) {
+        const int da = fx + i - ci.xa, db = ci.xb - fx - i;
+        r.set(i, (uint8_t)VT<uint8_t>::li_int(a, b, da, db, mg));
+      }
+    }
+  } else {
+#pragma unroll
+    for (int i = 0; i < N; ++i) {
+      const int da = fx + i - ci.xa, db = ci.xb - fx - i;
+      r.set(i, (!hb || da <= db) ? a : b);
+    }
+  }
+  return r;
+}
+
 // one sample at in-image column x of row rc.y (generic path: any x, any G)
 template <typename T, int SCHEME, int RECON>
-__device__ __forceinline__ T rebuild_px(const KParams& p, const Mask& m, const RowPlan& rp, const RowCtx& rc,
-                                        const T* ring, int slot_elems, int base, int x) {
-  using VTT = VT<T>;
+__device__ __noinline__ T rebuild_px(const KParams& p, const Mask& m, const RowPlan& rp, const RowCtx& rc,
+                                     const T* ring, int slot_elems, int base, int x) {
   const int col = x - base;
   if (SCHEME == S_NONE) return ring[rc.slot_c * slot_elems + col];
   if (SCHEME == S_ROW) {
     if (rc.kept) return ring[rc.slot_c * slot_elems + col];
-    const T a = rc.has_a ? ring[rc.slot_a * slot_elems + col] : T(0);
-    const T b = rc.has_b ? ring[rc.slot_b * slot_elems + col] : T(0);
-    if (RECON == R_LI && rc.has_a && rc.has_b) return VTT::li1(a, b, rc.da, rc.db);
-    return (!rc.has_b || (rc.has_a && rc.da <= rc.db)) ? a : b;
+    // (an NN-rebuilt row is marked kept with slot_a = the chosen loaded row)
+    const T a = ring[rc.slot_a * slot_elems + col];
+    const T b = ring[rc.slot_b * slot_elems + col];
+    if constexpr (sizeof(T) == 4) return fmaf(a - b, rc.wa, b);
+    else return li_px(a, b, rc.da, rc.db);
   }
   if (SCHEME == S_COL) {
     const int gx = x / p.G, t = gx % m.den;
     const T* row = ring + rc.slot_c * slot_elems;
     if (m.phase_kept(t)) return row[col];
     const int xa = (gx - m.dlo(t)) * p.G + p.G - 1;
-    int xb = (gx + m.dhi(t)) * p.G;
+    const int xb = (gx + m.dhi(t)) * p.G;
     const bool hb = xb <= p.W - 1;
     const int da = x - xa, db = xb - x;
     const T a = row[xa - base];
     const T b = hb ? row[xb - base] : T(0);
-    if (RECON == R_LI && hb) return VTT::li1(a, b, da, db);
+    if (RECON == R_LI && hb) return li_px(a, b, da, db);
     return (!hb || da <= db) ? a : b;
   }
-  // checker: rebuild along y in this column
-  int t = (x / p.G) % m.den + rc.ym;
+  int t = (x / p.G) % m.den + rc.ym;  // checker: rebuilt along y in this column
   if (t >= m.den) t -= m.den;
   if (m.phase_kept(t)) return ring[rc.slot_c * slot_elems + col];
   const int da = m.dlo(t), db = m.dhi(t);
@@ -341,70 +602,19 @@ __device__ __forceinline__ T rebuild_px(const KParams& p, const Mask& m, const R
   const bool ha = ya >= rp.lim_lo, hb = yb <= rp.lim_hi;
   const T a = ha ? ring[((ya - rp.lo) & (p.nr - 1)) * slot_elems + col] : T(0);
   const T b = hb ? ring[((yb - rp.lo) & (p.nr - 1)) * slot_elems + col] : T(0);
-  if (RECON == R_LI && ha && hb) return VTT::li1(a, b, da, db);
+  if (RECON == R_LI && ha && hb) return li_px(a, b, da, db);
   return (!hb || (ha && da <= db)) ? a : b;
 }
 
-// V samples of a chunk; out-of-image columns take the clamped column's sample
-// (clamp-to-edge addressing of the rebuilt image, R8)
-template <typename T, int SCHEME, int RECON>
-__device__ __forceinline__ typename VT<T>::Vec rebuild_chunk(const KParams& p, const Mask& m,
-                                                             const RowPlan& rp, const RowCtx& rc,
-                                                             const ChunkInfo& ci, const T* ring,
-                                                             int slot_elems, int base, int in_off) {
-  using VTT = VT<T>;
-  using Vec = typename VTT::Vec;
-  constexpr int V = VTT::V;
-  const int col = ci.xc - base;
-  if (ci.fast) {
-    if (SCHEME == S_NONE) return VTT::lds(ring + rc.slot_c * slot_elems + in_off + col);
-    if (SCHEME == S_ROW) {
-      if (rc.kept) return VTT::lds(ring + rc.slot_c * slot_elems + in_off + col);
-      if (RECON == R_LI && rc.has_a && rc.has_b)
-        return VTT::li_vec(VTT::lds(ring + rc.slot_a * slot_elems + in_off + col),
-                           VTT::lds(ring + rc.slot_b * slot_elems + in_off + col), rc.da, rc.db);
-      const int s = (!rc.has_b || (rc.has_a && rc.da <= rc.db)) ? rc.slot_a : rc.slot_b;
-      return VTT::lds(ring + s * slot_elems + in_off + col);
-    }
-    if (SCHEME == S_CHECKER) {
-      int t = ci.gxm + rc.ym;
-      if (t >= m.den) t -= m.den;
-      if (m.phase_kept(t)) return VTT::lds(ring + rc.slot_c * slot_elems + in_off + col);
-      const int da = m.dlo(t), db = m.dhi(t);
-      const int ya = rc.y - da, yb = rc.y + db;
-      const bool ha = ya >= rp.lim_lo, hb = yb <= rp.lim_hi;
-      const int sa = (ya - rp.lo) & (p.nr - 1), sb = (yb - rp.lo) & (p.nr - 1);
-      if (RECON == R_LI && ha && hb)
-        return VTT::li_vec(VTT::lds(ring + sa * slot_elems + in_off + col),
-                           VTT::lds(ring + sb * slot_elems + in_off + col), da, db);
-      const int s = (!hb || (ha && da <= db)) ? sa : sb;
-      return VTT::lds(ring + s * slot_elems + in_off + col);
-    }
-    // column scheme
-    const T* row = ring + rc.slot_c * slot_elems + in_off;
-    if (ci.col_kept) return VTT::lds(row + col);
-    const T a = row[ci.xa - base];
-    const bool hb = ci.xb >= 0;
-    const T b = hb ? row[ci.xb - base] : T(0);
-    Vec r;
+// generic path: N samples starting at column fx, each at the clamped column
+template <typename T, int N, int SCHEME, int RECON>
+__device__ __forceinline__ Frag<T, N> rebuild_frag_generic(const KParams& p, const Mask& m, const RowPlan& rp,
+                                                           const RowCtx& rc, const T* ring, int slot_elems,
+                                                           int fx, int base) {
+  Frag<T, N> r;
 #pragma unroll
-    for (int i = 0; i < V; ++i) {
-      const int da = ci.xc + i - ci.xa, db = ci.xb - ci.xc - i;
-      T v;
-      if (RECON == R_LI && hb) v = VTT::li1(a, b, da, db);
-      else v = (!hb || da <= db) ? a : b;
-      VTT::set(r, i, v);
-    }
-    return r;
-  }
-  // generic / edge path: per sample, clamped column
-  Vec r;
-  const T* ringo = ring + in_off;
-#pragma unroll
-  for (int i = 0; i < V; ++i) {
-    const int x = clampi(ci.xc + i, 0, p.W - 1);
-    VTT::set(r, i, rebuild_px<T, SCHEME, RECON>(p, m, rp, rc, ringo, slot_elems, base, x));
-  }
+  for (int i = 0; i < N; ++i)
+    r.set(i, rebuild_px<T, SCHEME, RECON>(p, m, rp, rc, ring, slot_elems, base, clampi(fx + i, 0, p.W - 1)));
   return r;
 }
 

@@ -8,30 +8,168 @@
 
 namespace kp {
 
-template <class App, int SCHEME, int RECON, int NCW>
-__global__ void __launch_bounds__(32 * (NCW + 1)) perf_kernel(const __grid_constant__ KParams p) {
+constexpr int kMaxVR = 3;  // largest vertical radius of an app (recipe table rows = seg_h + 2 VR)
+
+template <int I>
+struct IC {
+  static constexpr int value = I;
+};
+template <int I, int N, class F>
+__device__ __forceinline__ void static_for(F& f) {
+  if constexpr (I < N) {
+    f(IC<I>{});
+    static_for<I + 1, N>(f);
+  }
+}
+
+__device__ __forceinline__ void mbar_wait_u32(uint32_t addr, uint32_t parity) {
+  // watchdog: a protocol bug traps (launch error) instead of hanging the GPU
+  uint32_t ok, spins = 0;
+  do {
+    asm volatile(
+        "{\n .reg .pred p;\n mbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2;\n selp.u32 %0, 1, 0, p;\n}"
+        : "=r"(ok)
+        : "r"(addr), "r"(parity)
+        : "memory");
+    if (++spins > (1u << 26)) __trap();
+  } while (!ok);
+}
+__device__ __forceinline__ void mbar_arrive_u32(uint32_t addr) {
+  asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(addr) : "memory");
+}
+
+// (Ib) reconstruction + kernel execution of one work item for one consumer
+// warp.  FAST: every lane's V-chunk lies inside the image and in one mask cell.
+// ready / released are the warp's global (across items) ring counters.
+template <class App, int SCHEME, int RECON, int NCW, bool FAST>
+__device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int x0, int frame,
+                                         int ys, int ye, int g0, uint32_t full_u32, uint32_t empty_u32,
+                                         const typename App::T* ring, int slot_elems, const Recipe* rtab,
+                                         int& ready, int& released) {
   using T = typename App::T;
-  using VTT = VT<T>;
-  using Vec = typename VTT::Vec;
-  constexpr int V = VTT::V;
+  constexpr int V = App::V, EW = App::EW, VR = App::VR, NWIN = App::NWIN;
+  constexpr int CV = 16 / sizeof(T);  // elements of one 16-B mask-uniform chunk
+  const int lane = threadIdx.x & 31, w = (threadIdx.x >> 5) - 1;
+  const int xw = x0 + w * 32 * V;
+  const int base = x0 - p.hx;
+  const int xc = xw + lane * V;
+  const int ex = lane < 16 ? xw - EW : xw + 32 * V;  // edge fragment (warp halo) start column
+  const ChunkInfo cc = make_chunk<SCHEME>(p, m, xc);
+  const ChunkInfo ce = make_chunk<SCHEME>(p, m, lane < 16 ? xw - CV : xw + 32 * V);
+  // edge fragment: 0 inside the image, 1 left of column 0, 2 right of column W-1, 3 straddles W
+  const int emode = (ex >= 0 && ex + EW <= p.W) ? 0 : (ex < 0 ? 1 : (ex == p.W ? 2 : 3));
+  const int ccol = xc - base, ecol = ex - base;
+  const T* ring2 = ring + p.row_elems;  // second input (Hotspot power)
+  App app;
+  app.init(p);
+  T* optr = static_cast<T*>(p.out) + (long long)frame * p.out_fstride + (long long)(ys - p.out_row0) * p.W + xc;
+  const int nmask = p.nr - 1;
+  const int vy0 = ys - VR, vy1 = ye + VR;
+
+  auto step = [&](auto uc, int vy) {
+    constexpr int U = decltype(uc)::value;
+    const Recipe rec = rtab[vy - vy0];
+    const int need_hi = g0 + (rec.need & 0xFFFF), need_lo = g0 + (int)((uint32_t)rec.need >> 16);
+    // release ring slots no later row reads, then wait for the rows needed now
+#pragma unroll 1
+    while (released < need_lo) {
+      __syncwarp();
+      if (lane == 0) mbar_arrive_u32(empty_u32 + 8 * (released & nmask));
+      ++released;
+    }
+#pragma unroll 1
+    while (ready < need_hi) {
+      ++ready;
+      mbar_wait_u32(full_u32 + 8 * (ready & nmask), (ready >> p.nr_log2) & 1);
+    }
+    Frag<T, V> c, c2;
+    Frag<T, EW> e;
+    if (FAST) {
+      c = rebuild_frag<T, V, SCHEME, RECON>(p, m, rp, rec, cc, ring, slot_elems, ccol, xc, base);
+      if (App::NIN > 1) c2 = rebuild_frag<T, V, SCHEME, RECON>(p, m, rp, rec, cc, ring2, slot_elems, ccol, xc, base);
+      if (emode == 0) e = rebuild_frag<T, EW, SCHEME, RECON>(p, m, rp, rec, ce, ring, slot_elems, ecol, ex, base);
+      else if (emode == 1) e = Frag<T, EW>::splat(c.get(0));
+      else if (emode == 2) e = Frag<T, EW>::splat(c.get(V - 1));
+      else e = rebuild_frag_generic<T, EW, SCHEME, RECON>(p, m, rp, ctx_of<SCHEME>(rec), ring, slot_elems, ex, base);
+    } else {
+      const RowCtx rc = ctx_of<SCHEME>(rec);
+      c = rebuild_frag_generic<T, V, SCHEME, RECON>(p, m, rp, rc, ring, slot_elems, xc, base);
+      e = rebuild_frag_generic<T, EW, SCHEME, RECON>(p, m, rp, rc, ring, slot_elems, ex, base);
+      if (App::NIN > 1) c2 = rebuild_frag_generic<T, V, SCHEME, RECON>(p, m, rp, rc, ring2, slot_elems, xc, base);
+    }
+    const Frag<T, V> o = app.template row<U>(c, e, c2, lane, vy, xc, p);
+    if (vy >= ys + VR) {  // kernel execution result -> output buffer
+      if (FAST && p.vec_io) {
+#pragma unroll
+        for (int q = 0; q < (int)(V * sizeof(T)) / 16; ++q) {
+          const uint4 u = reinterpret_cast<const uint4*>(&o)[q];
+          st_global_v4(optr + q * CV, u.x, u.y, u.z, u.w);
+        }
+      } else {
+#pragma unroll
+        for (int i = 0; i < V; ++i)
+          if (FAST || xc + i < p.W) optr[i] = o.get(i);
+      }
+      optr += p.W;
+    }
+  };
+
+  for (int vb = vy0; vb < vy1; vb += NWIN) {
+    auto unrolled = [&](auto uc) {
+      const int vy = vb + decltype(uc)::value;
+      if (vy < vy1) step(uc, vy);
+    };
+    static_for<0, NWIN>(unrolled);
+  }
+  // every copy of this item lands, then its slots go back to the producer
+  const int g_end = g0 + rp.nload;
+#pragma unroll 1
+  while (ready < g_end - 1) {
+    ++ready;
+    mbar_wait_u32(full_u32 + 8 * (ready & nmask), (ready >> p.nr_log2) & 1);
+  }
+  __syncwarp();
+#pragma unroll 1
+  for (; released < g_end; ++released)
+    if (lane == 0) mbar_arrive_u32(empty_u32 + 8 * (released & nmask));
+}
+
+template <class App, int SCHEME, int RECON, int NCW>
+__device__ __forceinline__ void consumer_fast(const KParams& p, const Mask& m, const RowPlan& rp, int x0, int frame,
+                                              int ys, int ye, int g0, uint32_t full_u32, uint32_t empty_u32,
+                                              const typename App::T* ring, int slot_elems, const Recipe* rtab,
+                                              int& ready, int& released) {
+  consumer<App, SCHEME, RECON, NCW, true>(p, m, rp, x0, frame, ys, ye, g0, full_u32, empty_u32, ring, slot_elems,
+                                          rtab, ready, released);
+}
+template <class App, int SCHEME, int RECON, int NCW>
+__device__ __noinline__ void consumer_generic(const KParams& p, const Mask& m, const RowPlan& rp, int x0, int frame,
+                                              int ys, int ye, int g0, uint32_t full_u32, uint32_t empty_u32,
+                                              const typename App::T* ring, int slot_elems, const Recipe* rtab,
+                                              int& ready, int& released) {
+  consumer<App, SCHEME, RECON, NCW, false>(p, m, rp, x0, frame, ys, ye, g0, full_u32, empty_u32, ring, slot_elems,
+                                           rtab, ready, released);
+}
+
+// Persistent CTAs: CTA b processes work items b, b + gridDim.x, ...; an item is
+// (frame, segment of seg_h output rows, strip of TW columns), strip fastest.
+template <class App, int SCHEME, int RECON, int NCW>
+__global__ void __launch_bounds__(32 * (NCW + 1), App::MINB) perf_kernel(const __grid_constant__ KParams p) {
+  using T = typename App::T;
+  constexpr int V = App::V;
   constexpr int TW = NCW * 32 * V;
   extern __shared__ __align__(128) uint8_t smem[];
   uint64_t* full = reinterpret_cast<uint64_t*>(smem);
   uint64_t* empty = full + p.nr;
-  T* ring = reinterpret_cast<T*>(smem + ((2 * p.nr * 8 + 127) & ~127));
+  const int bar_bytes = (2 * p.nr * 8 + 127) & ~127;
+  T* ring = reinterpret_cast<T*>(smem + bar_bytes);
   const int slot_elems = p.row_elems * App::NIN;
-
-  int b = blockIdx.x;
-  const int strip = b % p.n_strips;
-  b /= p.n_strips;
-  const int seg = b % p.n_segs;
-  const int frame = b / p.n_segs;
-  const int x0 = strip * TW;
-  const int ys = p.y_begin + seg * p.seg_h;
-  const int ye = min(ys + p.seg_h, p.y_end);
-  const Mask m{p.num, p.den, p.keep_one};
-  const RowPlan rp = make_row_plan<SCHEME>(p, m, ys, ye, App::VR);
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  const int nrec = p.seg_h + 2 * kMaxVR;
+  Recipe* rtab = reinterpret_cast<Recipe*>(smem + bar_bytes + (size_t)p.nr * slot_elems * sizeof(T)) +
+                 (warp > 0 ? (warp - 1) * nrec : 0);  // one recipe table per consumer warp
+  const Mask m{p.num, p.den, p.keep_one};
+  const int n_items = p.n_strips * p.n_segs * p.frames;
 
   if (threadIdx.x == 0) {
     for (int s = 0; s < p.nr; ++s) {
@@ -41,105 +179,37 @@ __global__ void __launch_bounds__(32 * (NCW + 1)) perf_kernel(const __grid_const
     mbar_fence_init();
   }
   __syncthreads();
+  const uint32_t full_u32 = smem_u32(full), empty_u32 = smem_u32(empty);
 
-  if (warp == 0) {  // (Ia) data perforation: only kept samples leave HBM
-    producer<T, SCHEME, App::NIN, NCW>(p, m, rp, x0, frame, full, empty, ring);
-    return;
-  }
-
-  // ---------------- consumers: (Ib) reconstruction + kernel execution -------
-  const int w = warp - 1;
-  const int xw = x0 + w * 32 * V;
-  const int base = x0 - p.hx;
-  const int xc = xw + lane * V;
-  const ChunkInfo cc = make_chunk<SCHEME>(p, m, xc, V);
-  const ChunkInfo ce = make_chunk<SCHEME>(p, m, lane < 16 ? xw - V : xw + 32 * V, V);
-  App app;
-  app.init(p);
-  T* outp = static_cast<T*>(p.out) + (long long)frame * p.out_fstride;
-  const int nmask = p.nr - 1;
-
+  int g0 = 0;  // global load index of the current item's first row
   int ready = -1, released = 0;
-  int y_prev = -1, ym = 0, yq = 0;
-  for (int vy = ys - App::VR; vy < ye + App::VR; ++vy) {
-    const int y = clampi(vy, rp.lim_lo, rp.lim_hi);
-    if (y != y_prev) {  // y % den and y / den, incrementally
-      if (y_prev >= 0 && y == y_prev + 1) {
-        if (++ym == m.den) { ym = 0; ++yq; }
-      } else {
-        ym = y % m.den;
-        yq = y / m.den;
-      }
-      y_prev = y;
-    }
-    RowCtx rc;
-    rc.y = y;
-    rc.ym = ym;
-    rc.kept = 1;
-    rc.has_a = rc.has_b = 0;
-    rc.da = rc.db = 1;
-    rc.slot_a = rc.slot_b = 0;
-    int need_hi, need_lo;
-    if (SCHEME == S_ROW) {
-      rc.kept = m.phase_kept(ym);
-      if (rc.kept) {
-        const int id = (m.keep_one ? yq : yq * (m.den - 1) + ym) - rp.ord_lo;
-        rc.slot_c = id & nmask;
-        need_hi = need_lo = id;
-      } else {
-        rc.da = m.dlo(ym);
-        rc.db = m.dhi(ym);
-        rc.has_a = (y - rc.da) >= rp.lim_lo && (y - rc.da) >= rp.lo;
-        rc.has_b = (y + rc.db) <= rp.lim_hi && (y + rc.db) <= rp.hi;
-        const int ida = (m.keep_one ? yq : yq * (m.den - 1) + m.den - 2) - rp.ord_lo;
-        const int idb = (m.keep_one ? yq + 1 : (yq + 1) * (m.den - 1)) - rp.ord_lo;
-        rc.slot_a = ida & nmask;
-        rc.slot_b = idb & nmask;
-        rc.slot_c = rc.slot_a;
-        need_hi = rc.has_b ? idb : ida;
-        need_lo = rc.has_a ? ida : idb;
-      }
-    } else if (SCHEME == S_CHECKER) {
-      rc.slot_c = (y - rp.lo) & nmask;
-      need_hi = min(y + m.den - 1, rp.hi) - rp.lo;
-      need_lo = max(y - (m.den - 1), rp.lo) - rp.lo;
+  {
+    const int item = blockIdx.x;  // one work item per CTA (persistent variant)
+    if (item >= n_items) return;
+    int b = item;
+    const int strip = b % p.n_strips;
+    b /= p.n_strips;
+    const int seg = b % p.n_segs;
+    const int frame = b / p.n_segs;
+    const int x0 = strip * TW;
+    const int ys = p.y_begin + seg * p.seg_h;
+    const int ye = min(ys + p.seg_h, p.y_end);
+    const RowPlan rp = make_row_plan<SCHEME>(p, m, ys, ye, App::VR);
+    if (warp == 0) {  // (Ia) data perforation: only kept samples leave HBM
+      producer<T, SCHEME, App::NIN, TW>(p, m, rp, x0, frame, g0, full, empty, ring);
     } else {
-      rc.slot_c = (y - rp.lo) & nmask;
-      need_hi = need_lo = y - rp.lo;
-    }
-    // release ring slots no consumer row will read again, then wait for the rows needed now
-    if (released < need_lo) {
+      const int nv = ye - ys + 2 * App::VR;
       __syncwarp();
-      for (; released < need_lo; ++released)
-        if (lane == 0) mbar_arrive(&empty[released & nmask]);
+      for (int i = lane; i < nv; i += 32) rtab[i] = make_recipe<SCHEME, RECON>(p, m, rp, ys - App::VR + i);
+      __syncwarp();
+      const int xw = x0 + (warp - 1) * 32 * V;
+      if (p.fast_ok && xw + 32 * V <= p.W)
+        consumer_fast<App, SCHEME, RECON, NCW>(p, m, rp, x0, frame, ys, ye, g0, full_u32, empty_u32, ring,
+                                               slot_elems, rtab, ready, released);
+      else
+        consumer_generic<App, SCHEME, RECON, NCW>(p, m, rp, x0, frame, ys, ye, g0, full_u32, empty_u32, ring,
+                                                  slot_elems, rtab, ready, released);
     }
-    for (; ready < need_hi;) {
-      ++ready;
-      mbar_wait(&full[ready & nmask], (ready >> p.nr_log2) & 1);
-    }
-    const Vec c = rebuild_chunk<T, SCHEME, RECON>(p, m, rp, rc, cc, ring, slot_elems, base, 0);
-    const Vec e = rebuild_chunk<T, SCHEME, RECON>(p, m, rp, rc, ce, ring, slot_elems, base, 0);
-    Vec c2;
-    if (App::NIN > 1) c2 = rebuild_chunk<T, SCHEME, RECON>(p, m, rp, rc, cc, ring, slot_elems, base, p.row_elems);
-    else c2 = c;
-    const Vec o = app.row(c, e, c2, lane, vy, xc, p);
-    const int yo = vy - App::VR;
-    if (yo >= ys && xc < p.W) {  // kernel execution result -> output buffer
-      T* dst = outp + (long long)(yo - p.out_row0) * p.W + xc;
-      if (p.vec_io && xc + V <= p.W) {
-        const uint4 u = *reinterpret_cast<const uint4*>(&o);
-        st_global_v4(dst, u.x, u.y, u.z, u.w);
-      } else {
-#pragma unroll
-        for (int i = 0; i < V; ++i)
-          if (xc + i < p.W) dst[i] = VTT::get(o, i);
-      }
-    }
-  }
-  // every issued copy must land before the CTA retires
-  for (; ready < rp.nload - 1;) {
-    ++ready;
-    mbar_wait(&full[ready & nmask], (ready >> p.nr_log2) & 1);
   }
 }
 
@@ -150,9 +220,46 @@ cudaError_t launch_one(const KParams& p, unsigned grid, size_t smem, cudaStream_
   if (!attr) {
     cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, 227 * 1024);
     if (e != cudaSuccess) return e;
+    e = cudaFuncSetAttribute(k, cudaFuncAttributePreferredSharedMemoryCarveout, 100);  // max shared memory
+    if (e != cudaSuccess) return e;
     attr = true;
   }
-  k<<<grid, 32 * (NCW + 1), smem, s>>>(p);
+  // segment height: when not fixed by the caller (seg_auto), choose the number
+  // of row segments so the CTA count fills whole waves of resident CTA slots
+  // (occupancy API), discounted by the per-segment halo rows.
+  KParams q = p;
+  if (p.seg_auto) {
+    static int per_sm = 0, sms = 0;
+    static size_t per_sm_smem = 0;
+    if (per_sm == 0 || per_sm_smem != smem) {
+      int dev = 0;
+      cudaGetDevice(&dev);
+      cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
+      if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k, 32 * (NCW + 1), smem) != cudaSuccess ||
+          per_sm < 1)
+        per_sm = 1;
+      per_sm_smem = smem;
+    }
+    const long long slots = (long long)per_sm * sms;
+    const int rows = p.y_end - p.y_begin;
+    const long long per_seg = (long long)p.n_strips * p.frames;
+    double best = -1.0;
+    int best_n = (rows + p.seg_h - 1) / p.seg_h;
+    for (int n = (rows + p.seg_h - 1) / p.seg_h; n <= (rows + 31) / 32 && n <= 4 * best_n + 64; ++n) {
+      const int sh = (rows + n - 1) / n;
+      const int nn = (rows + sh - 1) / sh;
+      const long long items = per_seg * nn;
+      const long long waves = (items + slots - 1) / slots;
+      const double fill = (double)items / (double)(waves * slots);
+      const double halo = (double)sh / (double)(sh + 2 * App::VR + 2);
+      const double score = fill * halo;
+      if (score > best + 1e-9) { best = score; best_n = nn; }
+    }
+    q.seg_h = (rows + best_n - 1) / best_n;
+    q.n_segs = (rows + q.seg_h - 1) / q.seg_h;
+    grid = (unsigned)((long long)q.n_strips * q.n_segs * q.frames);
+  }
+  k<<<grid, 32 * (NCW + 1), smem, s>>>(q);
   return cudaGetLastError();
 }
 
@@ -181,6 +288,6 @@ cudaError_t launch_hotspot(int, int, const KParams&, unsigned, size_t, cudaStrea
 cudaError_t launch_gsobel(int, int, const KParams&, unsigned, size_t, cudaStream_t);
 cudaError_t launch_inversion(int, int, const KParams&, unsigned, size_t, cudaStream_t);
 
-constexpr int kNCW = 4;  // consumer warps per CTA (tile width 512 fp32 / 2048 u8 columns)
+constexpr int kNCW = 4;  // consumer warps per CTA (tile width 1024 fp32 / 4096 u8 columns)
 
 }  // namespace kp

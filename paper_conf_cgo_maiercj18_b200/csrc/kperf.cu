@@ -47,7 +47,7 @@ struct Band {  // banded Hotspot state
 struct perf_plan_s {
   int app, W, H, radius, scheme, recon;
   perf_rate rate;
-  long long batch = 1, iters = 1, granule_bytes = 32, global_h = -1, band_y0 = 0, tile_w = kp::kNCW, tile_h = 128,
+  long long batch = 1, iters = 1, granule_bytes = 128, global_h = -1, band_y0 = 0, tile_w = kp::kNCW, tile_h = 0,
             metric = 0, loader = 0, ring = 0;
   double* d_err = nullptr;
   float* d_tmp = nullptr;
@@ -78,7 +78,8 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
                                int in_row0, int avail0, int avail1, int out_row0, int y_begin, int y_end,
                                KParams& k, unsigned& grid, size_t& smem) {
   const int es = (int)elem_size(P->app);
-  const int V = 16 / es;
+  const int CV = 16 / es;  // elements per 16-B chunk (load / store / alignment unit)
+  const int V = P->app == PERF_APP_MEDIAN ? 16 : 8;  // elements per consumer lane per row (apps.cuh)
   const int NCW = kp::kNCW;
   const int TW = NCW * 32 * V;
   const int Hg = P->global_h > 0 ? (int)P->global_h : P->H;
@@ -104,41 +105,45 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   const int G = (int)(P->granule_bytes / es);
   k.G = G < 1 ? 1 : G;
   k.fast_ok = (scheme == PERF_SCHEME_NONE || scheme == PERF_SCHEME_ROW || (k.G % V) == 0) ? 1 : 0;
+  const bool chunk_uniform = scheme == PERF_SCHEME_NONE || scheme == PERF_SCHEME_ROW || (k.G % CV) == 0;
   const bool aligned = ((reinterpret_cast<uintptr_t>(in) | reinterpret_cast<uintptr_t>(out) |
                          reinterpret_cast<uintptr_t>(in2)) & 15) == 0;
-  k.vec_io = (P->W % V == 0) && aligned ? 1 : 0;
+  k.vec_io = (P->W % CV == 0) && aligned ? 1 : 0;
   int loader = (int)P->loader;
   if (loader == kp::L_AUTO) {
     if (!k.vec_io) loader = kp::L_SCALAR;
     else if (scheme == PERF_SCHEME_NONE || scheme == PERF_SCHEME_ROW) loader = kp::L_BULK;
-    else loader = k.fast_ok ? kp::L_ASYNC16 : kp::L_SCALAR;
+    else loader = chunk_uniform ? kp::L_ASYNC16 : kp::L_SCALAR;
   }
   if (loader == kp::L_BULK && !(k.vec_io && (scheme == PERF_SCHEME_NONE || scheme == PERF_SCHEME_ROW)))
     return fail(PERF_ERR_UNSUPPORTED, "loader BULK needs the row/none scheme, W % V == 0 and 16-B aligned buffers");
-  if (loader == kp::L_ASYNC16 && !(k.vec_io && k.fast_ok))
-    return fail(PERF_ERR_UNSUPPORTED, "loader ASYNC16 needs W % V == 0, aligned buffers and G % V == 0");
+  if (loader == kp::L_ASYNC16 && !(k.vec_io && chunk_uniform))
+    return fail(PERF_ERR_UNSUPPORTED, "loader ASYNC16 needs W*sizeof(T) % 16 == 0, aligned buffers, G*sizeof(T) % 16 == 0");
   k.loader = loader;
   // halo / apron columns: the lane edge chunk (V) plus, for the column scheme,
   // the distance to the nearest loaded granule on either side (<= den * G)
-  int hx = V;
-  if (scheme == PERF_SCHEME_COL) hx = ((V + k.den * k.G + V - 1) / V) * V;
+  int hx = CV;
+  if (scheme == PERF_SCHEME_COL) hx = ((CV + k.den * k.G + CV - 1) / CV) * CV;
   k.hx = hx;
   k.row_elems = TW + 2 * hx;
   // ring: rows a consumer holds for reconstruction + prefetch depth
   int hold = 1;
   if (scheme == PERF_SCHEME_ROW) hold = 2;
   if (scheme == PERF_SCHEME_CHECKER) hold = 2 * k.den - 1;
-  int nr = P->ring > 0 ? next_pow2((int)P->ring) : next_pow2(hold + 10);
+  int nr = P->ring > 0 ? next_pow2((int)P->ring) : next_pow2(hold + 6);
   if (nr < hold + 1) nr = next_pow2(hold + 1);
   const int nin = P->app == PERF_APP_HOTSPOT ? 2 : 1;
   const size_t slot_bytes = (size_t)k.row_elems * nin * es;
   auto bar_bytes = [](int n) { return (size_t)((2 * n * 8 + 127) & ~127); };
-  while (nr > next_pow2(hold + 1) && bar_bytes(nr) + nr * slot_bytes > 200 * 1024) nr >>= 1;
+  const size_t rec_bytes0 = (size_t)NCW * ((P->tile_h > 0 ? P->tile_h : 128) + 2 * kp::kMaxVR) * sizeof(kp::Recipe);
+  while (nr > next_pow2(hold + 1) && bar_bytes(nr) + nr * slot_bytes + rec_bytes0 > 200 * 1024) nr >>= 1;
   k.nr = nr;
   k.nr_log2 = log2i(nr);
-  smem = bar_bytes(nr) + (size_t)nr * slot_bytes;
-  if (smem > 227 * 1024) return fail(PERF_ERR_UNSUPPORTED, "shared-memory ring exceeds 227 KB");
   k.seg_h = (int)(P->tile_h > 0 ? P->tile_h : 128);
+  k.seg_auto = P->tile_h > 0 ? 0 : 1;
+  const size_t recipe_bytes = (size_t)NCW * (k.seg_h + 2 * kp::kMaxVR) * sizeof(kp::Recipe);
+  smem = bar_bytes(nr) + (size_t)nr * slot_bytes + recipe_bytes;
+  if (smem > 227 * 1024) return fail(PERF_ERR_UNSUPPORTED, "shared-memory ring + recipes exceed 227 KB");
   k.n_strips = (P->W + TW - 1) / TW;
   k.n_segs = (y_end - y_begin + k.seg_h - 1) / k.seg_h;
   k.frames = frames;
@@ -253,7 +258,7 @@ perf_status perf_plan_set(perf_plan_t p, int key, long long v) {
       p->tile_w = v;
       return PERF_OK;
     case PERF_KEY_TILE_H:
-      if (v < 1 || v > (1 << 20)) return fail(PERF_ERR_INVALID_ARG, "TILE_H out of range");
+      if (v < 1 || v > 4096) return fail(PERF_ERR_INVALID_ARG, "TILE_H must be in [1, 4096]");
       p->tile_h = v;
       return PERF_OK;
     case PERF_KEY_METRIC:

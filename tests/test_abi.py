@@ -49,7 +49,7 @@ def test_plan_validation(args, status):
 def test_plan_keys_roundtrip():
     h = kp.perf_plan("gaussian", 64, 48, 2, "col", (1, 4), "li")
     try:
-        assert kp.perf_plan_get(h, "granule_bytes") == 32
+        assert kp.perf_plan_get(h, "granule_bytes") == 128
         kp.perf_plan_set(h, "granule_bytes", 64)
         kp.perf_plan_set(h, "batch", 3)
         kp.perf_plan_set(h, "tile_h", 17)

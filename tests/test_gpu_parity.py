@@ -106,6 +106,28 @@ def test_granule_sizes(gbytes):
         assert_close("gaussian", 2, got, want)
 
 
+def test_default_granule_is_128_bytes():
+    """default cell width = the measured DRAM fill granule: 32 fp32 / 128 u8 pixels"""
+    W, H = 1536, 96
+    img = synth.image("natural", 21, W, H)
+    for scheme, rate, recon in [("col", (1, 2), "li"), ("checker", (1, 4), "nn"), ("col", (3, 4), "nn")]:
+        with kp.Plan("gaussian", W, H, 2, scheme, rate, recon) as p:
+            assert p.get("granule_bytes") == 128
+            x = torch.from_numpy(img).cuda()
+            y = torch.empty_like(x)
+            p.run(x, y)
+        want = oracle.run(oracle.params("gaussian", W, H, 2, scheme, rate, recon, 32), img)
+        assert_close("gaussian", 2, y.cpu().numpy(), want)
+    u = synth.image("natural", 22, 4096, 64, np.uint8)
+    for scheme, rate in [("col", (1, 2)), ("checker", (1, 2))]:
+        with kp.Plan("median", 4096, 64, 1, scheme, rate, "li") as p:
+            x = torch.from_numpy(u).cuda()
+            y = torch.empty_like(x)
+            p.run(x, y)
+        want = oracle.run(oracle.params("median", 4096, 64, 1, scheme, rate, "li", 128), u)
+        assert_close("median", 1, y.cpu().numpy(), want)
+
+
 @pytest.mark.parametrize("den", [2, 3, 5, 6, 7, 8])
 def test_all_denominators(den):
     W, H = 600, 90
@@ -161,7 +183,7 @@ def test_run_host_equals_run():
     W, H = 640, 96
     img = synth.image("natural", 4, W, H)
     out = np.zeros_like(img)
-    with kp.Plan("sobel", W, H, 1, "checker", (1, 2), "li") as p:
+    with kp.Plan("sobel", W, H, 1, "checker", (1, 2), "li", granule_bytes=32) as p:
         p.run_host(img, out)
     assert np.array_equal(out, gpu_run("sobel", 1, img, "checker", (1, 2), "li"))
 

@@ -1,0 +1,56 @@
+"""Launch selected perforated-stencil variants once each (for ncu captures).
+
+  python tools/ncu_driver.py [--config C2] [--variants all|headline|exact,...] [--batch B]
+
+Each variant: one warm-up launch on a separate buffer set is NOT done, so the
+k-th perf_kernel launch in the process is the k-th variant listed (ncu -k
+regex:perf_kernel -c N captures exactly the list).  Prints the order.
+"""
+import argparse
+import os
+import sys
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+sys.path.insert(0, ROOT)
+
+import torch  # noqa: E402
+
+import paper_conf_cgo_maiercj18_b200 as kp  # noqa: E402
+import synth  # noqa: E402
+
+
+def variants(which):
+    out = []
+    for app, r in (("gaussian", 2), ("sobel", 1)):
+        out.append((app, r, "none", (0, 1), "nn"))
+        for s in ("row", "col", "checker"):
+            for rate in ((1, 2), (1, 4), (3, 4)):
+                for rc in ("nn", "li"):
+                    out.append((app, r, s, rate, rc))
+    if which == "all":
+        return out
+    if which == "headline":
+        return [("gaussian", 2, "row", (1, 2), "li"), ("gaussian", 2, "none", (0, 1), "nn")]
+    return [v for v in out if f"{v[0]}{v[1]}_{v[2]}_{v[3][0]}-{v[3][1]}_{v[4]}" in which.split(",")]
+
+
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--variants", default="all")
+    ap.add_argument("--batch", type=int, default=2)
+    ap.add_argument("--gran", type=int, default=32)
+    a = ap.parse_args()
+    W = H = 4096
+    x = torch.empty((a.batch, H, W), device="cuda")
+    synth.image_device("natural", 0x5EED0011, W, H, a.batch, x.data_ptr(), False)
+    y = torch.empty_like(x)
+    torch.cuda.synchronize()
+    for app, r, s, rate, rc in variants(a.variants):
+        with kp.Plan(app, W, H, r, s, rate, rc, batch=a.batch, granule_bytes=a.gran) as p:
+            p.run(x, y)
+            torch.cuda.synchronize()
+        print(f"{app}{r}_{s}_{rate[0]}-{rate[1]}_{rc}", flush=True)
+
+
+if __name__ == "__main__":
+    main()
