@@ -51,7 +51,7 @@ __device__ __forceinline__ float deriv(const float* x) {
 template <int R>
 struct AppGauss {  // K1 Gaussian, binomial (2R+1)^2, fp32
   using T = float;
-  static constexpr int V = 8, EW = 2, VR = R, NIN = 1, NWIN = 2 * R + 1, MINB = 1;
+  static constexpr int V = 8, EW = 2, VR = R, NIN = 1, NWIN = 2 * R + 1, MINB = 4;
   f2 h[NWIN][V / 2];  // horizontal results, column pairs (FADD2/FFMA2 vertical pass)
   __device__ void init(const KParams&) {}
   template <int U>
@@ -80,7 +80,7 @@ struct AppGauss {  // K1 Gaussian, binomial (2R+1)^2, fp32
 template <int R>
 struct AppSobel {  // K5 Sobel, |(Gx, Gy)|, fp32
   using T = float;
-  static constexpr int V = 8, EW = 2, VR = R, NIN = 1, NWIN = 2 * R + 1, MINB = 1;
+  static constexpr int V = 8, EW = 2, VR = R, NIN = 1, NWIN = 2 * R + 1, MINB = R == 1 ? 4 : 3;
   f2 sx[NWIN][V / 2], dx[NWIN][V / 2];  // horizontal smoothing / derivative, column pairs
   __device__ void init(const KParams&) {}
   template <int U>
@@ -121,7 +121,7 @@ struct AppSobel {  // K5 Sobel, |(Gx, Gy)|, fp32
 
 struct AppInversion {  // K2 Inversion, 255 - x
   using T = float;
-  static constexpr int V = 8, EW = 2, VR = 0, NIN = 1, NWIN = 1, MINB = 1;
+  static constexpr int V = 8, EW = 2, VR = 0, NIN = 1, NWIN = 1, MINB = 4;
   __device__ void init(const KParams&) {}
   template <int U>
   __device__ __forceinline__ Frag<float, V> row(const Frag<float, V>& c, const Frag<float, EW>&,
@@ -137,7 +137,7 @@ struct AppInversion {  // K2 Inversion, 255 - x
 // K4 Hotspot (Rodinia 2D transient thermal step), T and P rebuilt alike.
 struct AppHotspot {
   using T = float;
-  static constexpr int V = 8, EW = 2, VR = 1, NIN = 2, NWIN = 3, MINB = 1;
+  static constexpr int V = 8, EW = 2, VR = 1, NIN = 2, NWIN = 3, MINB = 4;
   float tc[3][V], tl[3], tr[3], pc[3][V];
   float sdc, rx1, ry1, rz1, amb;
   __device__ void init(const KParams& p) {
@@ -177,7 +177,7 @@ struct AppHotspot {
 // registers; Sobel clamps in the Gaussian image (G(-1) = G(0), G(W) = G(W-1)).
 struct AppGaussSobel {
   using T = float;
-  static constexpr int V = 8, EW = 4, VR = 3, NIN = 1, NWIN = 1, MINB = 1;
+  static constexpr int V = 8, EW = 4, VR = 3, NIN = 1, NWIN = 1, MINB = 3;
   float h[5][V + 1];   // horizontal Gaussian of the last 5 input rows: V lane columns + 1 edge column
   float gs[3][V + 2];  // last 3 Gaussian rows, lane columns -1..V
   __device__ void init(const KParams&) {}
@@ -274,7 +274,7 @@ struct AppGaussSobel {
 // on packed u16x2 lanes (VIMNMX.U16x2), 2 pixels per instruction.
 struct AppMedian {
   using T = uint8_t;
-  static constexpr int V = 16, EW = 4, VR = 1, NIN = 1, NWIN = 3, MINB = 1;
+  static constexpr int V = 16, EW = 4, VR = 1, NIN = 1, NWIN = 3, MINB = 3;
   static constexpr int NW = V / 2 + 2;  // u16x2 words per row incl. the two halo words
   uint32_t r[3][NW];  // word 0 = (_, col -1), words 1..V/2 = cols 0..V-1, last = (col V, _)
   __device__ void init(const KParams&) {}

@@ -542,13 +542,10 @@ __device__ __forceinline__ Frag<T, N> rebuild_frag(const KParams& p, const Mask&
   const T b = hb ? row[ci.xb - base] : a;
   Frag<T, N> r;
   if (RECON == R_LI && hb) {
-    if constexpr (sizeof(T) == 4) {
-      const float inv = __frcp_rn((float)(ci.xb - ci.xa));
+    if constexpr (sizeof(T) == 4) {  // b + (a - b) * (xb - x) / (xb - xa)
+      const float inv = __frcp_rn((float)(ci.xb - ci.xa)), d = a - b, x0 = (float)(ci.xb - fx);
 #pragma unroll
-      for (int i = 0; i < N; ++i) {
-        const int da = fx + i - ci.xa, db = ci.xb - fx - i;
-        r.set(i, VT<float>::li(a, b, (float)da, (float)db, inv));
-      }
+      for (int i = 0; i < N; ++i) r.set(i, fmaf(d, __fmul_rn(x0 - (float)i, inv), b));
     } else {
       const uint32_t mg = VT<uint8_t>::magic_of(ci.xb - ci.xa);
 #pragma unroll
@@ -557,11 +554,21 @@ __device__ __forceinline__ Frag<T, N> rebuild_frag(const KParams& p, const Mask&
         r.set(i, (uint8_t)VT<uint8_t>::li_int(a, b, da, db, mg));
       }
     }
-  } else {
+  } else {  // nearest: a while 2x <= xa + xb (ties to the lower column)
+    const int lim = ci.xa + ci.xb - 2 * fx;
+    if constexpr (sizeof(T) == 1) {  // per-byte select with word masks
+      const uint32_t wa = 0x01010101u * a, wb = 0x01010101u * b;
 #pragma unroll
-    for (int i = 0; i < N; ++i) {
-      const int da = fx + i - ci.xa, db = ci.xb - fx - i;
-      r.set(i, (!hb || da <= db) ? a : b);
+      for (int k = 0; k < N / 4; ++k) {
+        uint32_t msk = 0;
+#pragma unroll
+        for (int j = 0; j < 4; ++j)
+          if (!hb || 2 * (4 * k + j) <= lim) msk |= 0xFFu << (8 * j);
+        r.w[k] = (wa & msk) | (wb & ~msk);
+      }
+    } else {
+#pragma unroll
+      for (int i = 0; i < N; ++i) r.set(i, (!hb || 2 * i <= lim) ? a : b);
     }
   }
   return r;
@@ -591,7 +598,11 @@ __device__ __noinline__ T rebuild_px(const KParams& p, const Mask& m, const RowP
     const int da = x - xa, db = xb - x;
     const T a = row[xa - base];
     const T b = hb ? row[xb - base] : T(0);
-    if (RECON == R_LI && hb) return li_px(a, b, da, db);
+    if (RECON == R_LI && hb) {
+      if constexpr (sizeof(T) == 4)  // same arithmetic as the fast path
+        return fmaf(a - b, __fmul_rn((float)db, __frcp_rn((float)(xb - xa))), b);
+      else return li_px(a, b, da, db);
+    }
     return (!hb || da <= db) ? a : b;
   }
   int t = (x / p.G) % m.den + rc.ym;  // checker: rebuilt along y in this column

@@ -171,14 +171,21 @@ __global__ void __launch_bounds__(32 * (NCW + 1), App::MINB) perf_kernel(const _
   const Mask m{p.num, p.den, p.keep_one};
   const int n_items = p.n_strips * p.n_segs * p.frames;
 
+  // consumer warps whose columns all lie right of the image have nothing to do
+  int nact = NCW;
+  {
+    const int x0s = (blockIdx.x % p.n_strips) * TW;
+    nact = min(NCW, (p.W - x0s + 32 * V - 1) / (32 * V));
+  }
   if (threadIdx.x == 0) {
     for (int s = 0; s < p.nr; ++s) {
       mbar_init(&full[s], p.loader == L_BULK ? 1u : 32u);
-      mbar_init(&empty[s], (uint32_t)NCW);
+      mbar_init(&empty[s], (uint32_t)nact);
     }
     mbar_fence_init();
   }
   __syncthreads();
+  if (warp > nact) return;
   const uint32_t full_u32 = smem_u32(full), empty_u32 = smem_u32(empty);
 
   int g0 = 0;  // global load index of the current item's first row

@@ -239,7 +239,7 @@ def test_hotspot_parity(scheme, rate, recon, iters):
     T, P = synth.hotspot(synth.SEED_C4, W, H)
     Td, Pd = torch.from_numpy(T).cuda(), torch.from_numpy(P).cuda()
     out = torch.empty_like(Td)
-    with kp.Plan("hotspot", W, H, 1, scheme, rate, recon, iters=iters) as p:
+    with kp.Plan("hotspot", W, H, 1, scheme, rate, recon, iters=iters, granule_bytes=32) as p:
         p.hotspot(Td, Pd, out)
         torch.cuda.synchronize()
     want = oracle.hotspot(oracle.params("hotspot", W, H, 1, scheme, rate, recon, 8), T, P, iters)
