@@ -414,7 +414,7 @@ def bench_hotspot(args, cfg, ws, rank, local, stream, peak, peak_src):
     import synth
     W, Hg, iters = cfg["W"], cfg["H"], cfg["iters"]
     # row bands: rank k owns rows [y0, y0 + h)
-    cuts = [Hg * i // ws for i in range(ws + 1)]
+    cuts = kp.band_cuts(Hg, ws)
     y0, h = cuts[rank], cuts[rank + 1] - cuts[rank]
     T = torch.empty((h, W), device="cuda")
     P = torch.empty((h, W), device="cuda")

@@ -94,7 +94,8 @@ enum {
   PERF_KEY_TILE_H = 7,         /* output rows per CTA segment (default 128) */
   PERF_KEY_METRIC = 8,         /* perf_metric used by perf_error (default: MRE; ME for Sobel apps) */
   PERF_KEY_LOADER = 9,         /* 0 auto, 1 TMA bulk rows, 2 cp.async 16 B, 3 scalar (any alignment) */
-  PERF_KEY_RING = 10           /* shared-memory ring depth in rows (0 = auto) */
+  PERF_KEY_RING = 10,          /* shared-memory ring depth in rows (0 = auto) */
+  PERF_KEY_HALO_ROWS = 11      /* read-only: rows a Hotspot band exchanges with each neighbour per step */
 };
 
 /* Create a plan.  Validates: W, H >= 1; radius allowed for the app (Gaussian,

@@ -68,6 +68,7 @@ def lib():
             "orc_hotspot_coeffs": (None, [vp, vp, vp, vp, vp]),
             "orc_hotspot_run": (None, [P, vp, vp, i, vp]),
             "orc_hotspot_rect": (None, [P, vp, vp, i, i, i, i, i, vp]),
+            "orc_hotspot_window": (None, [P, vp, vp, i, i, i, i, i]),
             "orc_error_f64": (d, [i, vp, vp, ll, vp]),
             "orc_error_f32": (d, [i, vp, vp, ll, vp]),
             "orc_error_u8": (d, [i, vp, vp, ll, vp]),
@@ -155,6 +156,14 @@ def hotspot_rect(p: OrcParams, T0, P, iters, x0, y0, w, h) -> np.ndarray:
     out = np.zeros((h, w), dtype=np.float64)
     lib().orc_hotspot_rect(ctypes.byref(p), _ptr(T0), _ptr(P), iters, x0, y0, w, h, _ptr(out))
     return out
+
+
+def hotspot_window(p: OrcParams, T: np.ndarray, P: np.ndarray, ox: int, oy: int, iters: int) -> None:
+    """iters steps in place on a window (fp64 T, fp32 P) whose pixel (0,0) is global (ox, oy)"""
+    assert T.dtype == np.float64 and T.flags["C_CONTIGUOUS"] and T.shape == P.shape
+    P = np.ascontiguousarray(P, dtype=np.float32)
+    h, w = T.shape
+    lib().orc_hotspot_window(ctypes.byref(p), _ptr(T), _ptr(P), ox, oy, w, h, iters)
 
 
 def error(metric: str, exact: np.ndarray, approx: np.ndarray):

@@ -319,6 +319,12 @@ static void hotspot_window(const orc_params* p, double* T, const float* P, int o
   free(Pr);
 }
 
+/* iters steps on a caller-owned window (global origin ox, oy; w x h) -- the
+ * building block of the band-decomposition test (tests/test_multirank_cpu.py) */
+void orc_hotspot_window(const orc_params* p, double* T, const float* P, int ox, int oy, int w, int h, int iters) {
+  hotspot_window(p, T, P, ox, oy, w, h, iters);
+}
+
 void orc_hotspot_run(const orc_params* p, const float* T0, const float* P, int iters, double* Tout) {
   const long long n = (long long)p->W * p->H;
   for (long long i = 0; i < n; ++i) Tout[i] = (double)T0[i];

@@ -55,6 +55,10 @@ int orc_run_pixel_u8(const orc_params* p, const uint8_t* in, int x, int y);
  * perforated and rebuilt every step. */
 void orc_hotspot_coeffs(double* step_div_cap, double* rx_1, double* ry_1, double* rz_1, double* amb);
 void orc_hotspot_run(const orc_params* p, const float* T0, const float* P, int iters, double* Tout);
+/* iters steps on a window of the global grid (origin ox, oy; w x h); T is
+ * fp64 in/out, P fp32; values near window edges that are not image edges
+ * are invalid after the steps (outside the dependency cone). */
+void orc_hotspot_window(const orc_params* p, double* T, const float* P, int ox, int oy, int w, int h, int iters);
 /* final temperature on the rectangle [x0,x0+w) x [y0,y0+h) only, computed on
  * the dependency cone (same result as orc_hotspot_run restricted to it). */
 void orc_hotspot_rect(const orc_params* p, const float* T0, const float* P, int iters, int x0, int y0,

@@ -22,7 +22,7 @@ SCHEME = {"none": 0, "row": 1, "col": 2, "checker": 3}
 RECON = {"nn": 0, "li": 1, "linear": 1}
 METRIC = {"mre": 0, "me": 1, "mae": 2}
 KEY = {"batch": 1, "iters": 2, "granule_bytes": 3, "global_h": 4, "band_y0": 5, "tile_w": 6, "tile_h": 7,
-       "metric": 8, "loader": 9, "ring": 10}
+       "metric": 8, "loader": 9, "ring": 10, "halo_rows": 11}
 STATUS = {0: "PERF_OK", 1: "PERF_ERR_INVALID_ARG", 2: "PERF_ERR_UNSUPPORTED", 3: "PERF_ERR_CUDA",
           4: "PERF_ERR_NCCL", 5: "PERF_ERR_OOM"}
 
@@ -167,6 +167,13 @@ def perf_comm_init(plan: int, unique_id: bytes, rank: int, nranks: int) -> None:
 
 def perf_destroy(plan: int) -> None:
     _check(lib().perf_destroy(plan))
+
+
+def band_cuts(H: int, nranks: int):
+    """Row bands of a sharded Hotspot grid: rank k owns rows [cuts[k], cuts[k+1])."""
+    if nranks < 1 or H < nranks:
+        raise ValueError("need 1 <= nranks <= H")
+    return [H * k // nranks for k in range(nranks + 1)]
 
 
 class Plan:

@@ -185,6 +185,13 @@ static cudaError_t dispatch(const perf_plan_s* P, const KParams& k, unsigned gri
   return cudaErrorInvalidValue;
 }
 
+static int band_halo(const perf_plan_s* p) {
+  // stencil radius 1 + distance to the loaded rows a rebuilt row reads
+  const bool vertical = p->rate.num > 0 && (p->scheme == PERF_SCHEME_ROW || p->scheme == PERF_SCHEME_CHECKER);
+  return 1 + (vertical ? p->rate.den : 0);
+}
+
+
 extern "C" {
 
 const char* perf_last_error(void) { return g_err.c_str(); }
@@ -273,6 +280,8 @@ perf_status perf_plan_set(perf_plan_t p, int key, long long v) {
       if (v < 0 || v > 256) return fail(PERF_ERR_INVALID_ARG, "bad RING");
       p->ring = v;
       return PERF_OK;
+    case PERF_KEY_HALO_ROWS:
+      return fail(PERF_ERR_INVALID_ARG, "HALO_ROWS is read-only");
   }
   return fail(PERF_ERR_INVALID_ARG, "unknown key");
 }
@@ -290,6 +299,7 @@ perf_status perf_plan_get(perf_plan_t p, int key, long long* v) {
     case PERF_KEY_METRIC: *v = p->metric; return PERF_OK;
     case PERF_KEY_LOADER: *v = p->loader; return PERF_OK;
     case PERF_KEY_RING: *v = p->ring; return PERF_OK;
+    case PERF_KEY_HALO_ROWS: *v = band_halo(p); return PERF_OK;
   }
   return fail(PERF_ERR_INVALID_ARG, "unknown key");
 }
@@ -331,12 +341,6 @@ perf_status perf_run_host(perf_plan_t p, const void* host_in, void* host_out, vo
 }
 
 // ---------------------------------------------------------------- Hotspot ----
-static int band_halo(const perf_plan_s* p) {
-  // stencil radius 1 + distance to the loaded rows a rebuilt row reads
-  const bool vertical = p->rate.num > 0 && (p->scheme == PERF_SCHEME_ROW || p->scheme == PERF_SCHEME_CHECKER);
-  return 1 + (vertical ? p->rate.den : 0);
-}
-
 static perf_status band_alloc(perf_plan_s* p) {
   const int hb = band_halo(p);
   const size_t rows = (size_t)p->H + 2 * hb;
