@@ -86,6 +86,38 @@ def ncu_traffic(kernel_key):
         return None
 
 
+_bwp = None
+_mix_cache = {}
+
+
+def mixed_peak_gbs(in_ptr, out_ptr, out_bytes, scheme, rate, gran_bytes=128, n_in=1, stream=0):
+    """GB/s a plain streaming kernel reaches with the same read/write mix as a
+    perforated stencil (tools/bwprobe.cu, measured on this box): every output
+    byte written once, the kept fraction of the input read, in 16-KB rows (row
+    scheme / exact) or gran_bytes cells (column / checker).  Algorithmic bytes
+    over the probe's time, so it is directly comparable to roofline.achieved."""
+    global _bwp
+    import ctypes
+    if _bwp is None:
+        _bwp = ctypes.CDLL(os.path.join(ROOT, "tools", "libbwprobe.so"))
+        _bwp.bwp_time_ms.restype = ctypes.c_float
+        _bwp.bwp_time_ms.argtypes = [ctypes.c_void_p, ctypes.c_void_p, ctypes.c_longlong, ctypes.c_int,
+                                     ctypes.c_int, ctypes.c_int, ctypes.c_int, ctypes.c_int, ctypes.c_void_p]
+    num, den = rate
+    if scheme == "none" or num == 0:
+        kn, kd = 1, 1
+    else:
+        kd = den
+        kn = den - num
+    unit = 16384 if scheme in ("none", "row") else gran_bytes
+    key = (out_bytes, kn, kd, unit, n_in)
+    if key not in _mix_cache:
+        ms = _bwp.bwp_time_ms(in_ptr, out_ptr, out_bytes, kn, kd, unit, n_in, 5, stream)
+        k = kn / kd
+        _mix_cache[key] = (n_in * k + 1.0) * out_bytes / (ms * 1e-3) / 1e9 if ms > 0 else None
+    return _mix_cache[key]
+
+
 class ClockSampler:
     FIELDS = ("clocks.sm,clocks.max.sm,power.draw,clocks_event_reasons.hw_slowdown,"
               "clocks_event_reasons.hw_thermal_slowdown,clocks_event_reasons.sw_thermal_slowdown,"
@@ -320,6 +352,8 @@ def main():
         achieved = algo_b / (ms * 1e-3) / 1e9
         kkey = f"{app}{cfg['r']}_{cfg['scheme']}_{cfg['rate'][0]}-{cfg['rate'][1]}_{cfg['recon']}"
         tr = ncu_traffic(kkey)
+        pmix = mixed_peak_gbs(x.data_ptr(), yex.data_ptr(), px_step * es, cfg["scheme"], cfg["rate"], G,
+                              stream=stream.cuda_stream) if not u8 else None
         result = {
             "metric": METRIC, "value": value, "unit": unit, "n_gpus": ws, "steps": args.steps,
             "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True, "scaling": "weak",
@@ -334,7 +368,9 @@ def main():
             "hbm_gbs": achieved,
             "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
                          "frac": achieved / peak, "traffic": tr, "kernel": kkey,
-                         "algorithmic_bytes_per_launch": algo_b, "peak_source": peak_src},
+                         "algorithmic_bytes_per_launch": algo_b, "peak_source": peak_src,
+                         "peak_mix": pmix, "frac_mix": achieved / pmix if pmix else None,
+                         "peak_mix_source": "tools/bwprobe.cu on this box: plain stream, same read/write mix"},
             "clocks": clk.summary(),
             "gpu_launches": args.steps,
         }
@@ -388,9 +424,11 @@ def bench_variants(kp, cfg, x, y, yex, stream, peak, ws):
     for app, r in (("gaussian", 2), ("sobel", 1)):
         ex = kp.Plan(app, W, H, r, "none", (0, 1), "nn", batch=B)
         ms_ex = time_kernel(lambda: ex.run(x, yex, stream), stream, 10, 3)
+        pm_ex = mixed_peak_gbs(x.data_ptr(), y.data_ptr(), px * 4, "none", (0, 1), 128, stream=stream.cuda_stream)
         out.append({"app": app, "r": r, "scheme": "none", "rate": [0, 1], "recon": "-", "ms": ms_ex,
                     "mpixel_s": px / ms_ex / 1e3, "speedup": 1.0, "error": 0.0,
-                    "hbm_gbs": 8 * px / ms_ex / 1e6, "frac": 8 * px / ms_ex / 1e6 / peak})
+                    "hbm_gbs": 8 * px / ms_ex / 1e6, "frac": 8 * px / ms_ex / 1e6 / peak,
+                    "frac_mix": 8 * px / ms_ex / 1e6 / pm_ex if pm_ex else None})
         for scheme in ("row", "col", "checker"):
             for rate in ((1, 2), (1, 4), (3, 4)):
                 for recon in ("nn", "li"):
@@ -398,10 +436,16 @@ def bench_variants(kp, cfg, x, y, yex, stream, peak, ws):
                     ms = time_kernel(lambda: p.run(x, y, stream), stream, 10, 3)
                     err, _ = p.error(yex, y, stream)
                     gbs = bytes_per_px(app, scheme, rate) * px / ms / 1e6
+                    pm = mixed_peak_gbs(x.data_ptr(), y.data_ptr(), px * 4, scheme, rate, 128,
+                                        stream=stream.cuda_stream)
+                    pm_ex = mixed_peak_gbs(x.data_ptr(), y.data_ptr(), px * 4, "none", (0, 1), 128,
+                                           stream=stream.cuda_stream)
                     out.append({"app": app, "r": r, "scheme": scheme, "rate": list(rate), "recon": recon,
                                 "ms": ms, "mpixel_s": px / ms / 1e3, "speedup": ms_ex / ms, "error": err,
-                                "hbm_gbs": gbs, "frac": gbs / peak,
-                                "ceiling": (8.0) / bytes_per_px(app, scheme, rate)})
+                                "hbm_gbs": gbs, "frac": gbs / peak, "frac_mix": gbs / pm if pm else None,
+                                "byte_ceiling": 8.0 / bytes_per_px(app, scheme, rate),
+                                "mix_ceiling": (pm / bytes_per_px(app, scheme, rate)) / (pm_ex / 8.0)
+                                if pm and pm_ex else None})
                     p.close()
         ex.close()
     return out
@@ -453,6 +497,10 @@ def bench_hotspot(args, cfg, ws, rank, local, stream, peak, peak_src):
     cells = W * Hg * iters
     algo_b = bytes_per_px("hotspot", cfg["scheme"], cfg["rate"]) * W * h * iters
     achieved = algo_b / (ms * 1e-3) / 1e9
+    scratch = torch.empty((2, h, W), device="cuda")
+    pmix = mixed_peak_gbs(scratch.data_ptr(), out_ex.data_ptr(), W * h * 4, cfg["scheme"], cfg["rate"], 128,
+                          n_in=2, stream=stream.cuda_stream)
+    del scratch
     return {"metric": METRIC, "value": cells / (ms * 1e-3) / 1e6, "unit": "Mcell-updates/s", "n_gpus": ws,
             "steps": args.steps, "warmup": 1, "ms_per_step": ms, "higher_is_better": True,
             "scaling": "strong", "vs_baseline": None, "dtype": "f32", "data": "synthetic",
@@ -460,7 +508,8 @@ def bench_hotspot(args, cfg, ws, rank, local, stream, peak, peak_src):
                        else "none"},
             "speedup_vs_exact": ms_ex / ms, "error": {"metric": "mre", "value": mre, "count": cnt},
             "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
-                         "frac": achieved / peak, "traffic": None, "peak_source": peak_src},
+                         "frac": achieved / peak, "traffic": None, "peak_source": peak_src,
+                         "peak_mix": pmix, "frac_mix": achieved / pmix if pmix else None},
             "clocks": clk.summary(), "gpu_launches": args.steps * iters}
 
 

@@ -14,7 +14,7 @@ import ctypes
 import os
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
-LIB_PATH = os.path.join(_HERE, "libkperf.so")
+LIB_PATH = os.environ.get("KPERF_LIB", os.path.join(_HERE, "libkperf.so"))  # override: experiment builds
 
 # enums (mirror include/kperf.h)
 APP = {"gaussian": 0, "sobel": 1, "median": 2, "hotspot": 3, "gauss_sobel": 4, "inversion": 5}

@@ -6,6 +6,13 @@
 #include "apps.cuh"
 #include "engine.cuh"
 
+#ifndef KPERF_PIPELINE
+#define KPERF_PIPELINE 0
+#endif
+#ifndef KPERF_MINB
+#define KPERF_MINB 0  // 0: per-app App::MINB
+#endif
+
 namespace kp {
 
 constexpr int kMaxVR = 3;  // largest vertical radius of an app (recipe table rows = seg_h + 2 VR)
@@ -66,11 +73,16 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
   const int nmask = p.nr - 1;
   const int vy0 = ys - VR, vy1 = ye + VR;
 
-  auto step = [&](auto uc, int vy) {
-    constexpr int U = decltype(uc)::value;
+  struct Rows {  // one rebuilt input row as the lane sees it
+    Frag<T, V> c, c2;
+    Frag<T, EW> e;
+  };
+  // fetch: recipe, ring release/wait, rebuild from shared memory (a1/a2)
+  auto fetch = [&](int vy) {
+    Rows r;
     const Recipe rec = rtab[vy - vy0];
     const int need_hi = g0 + (rec.need & 0xFFFF), need_lo = g0 + (int)((uint32_t)rec.need >> 16);
-    // release ring slots no later row reads, then wait for the rows needed now
+    // release ring slots no later row reads (earlier rows are already in registers)
 #pragma unroll 1
     while (released < need_lo) {
       __syncwarp();
@@ -82,22 +94,25 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
       ++ready;
       mbar_wait_u32(full_u32 + 8 * (ready & nmask), (ready >> p.nr_log2) & 1);
     }
-    Frag<T, V> c, c2;
-    Frag<T, EW> e;
     if (FAST) {
-      c = rebuild_frag<T, V, SCHEME, RECON>(p, m, rp, rec, cc, ring, slot_elems, ccol, xc, base);
-      if (App::NIN > 1) c2 = rebuild_frag<T, V, SCHEME, RECON>(p, m, rp, rec, cc, ring2, slot_elems, ccol, xc, base);
-      if (emode == 0) e = rebuild_frag<T, EW, SCHEME, RECON>(p, m, rp, rec, ce, ring, slot_elems, ecol, ex, base);
-      else if (emode == 1) e = Frag<T, EW>::splat(c.get(0));
-      else if (emode == 2) e = Frag<T, EW>::splat(c.get(V - 1));
-      else e = rebuild_frag_generic<T, EW, SCHEME, RECON>(p, m, rp, ctx_of<SCHEME>(rec), ring, slot_elems, ex, base);
+      r.c = rebuild_frag<T, V, SCHEME, RECON>(p, m, rp, rec, cc, ring, slot_elems, ccol, xc, base);
+      if (App::NIN > 1) r.c2 = rebuild_frag<T, V, SCHEME, RECON>(p, m, rp, rec, cc, ring2, slot_elems, ccol, xc, base);
+      if (emode == 0) r.e = rebuild_frag<T, EW, SCHEME, RECON>(p, m, rp, rec, ce, ring, slot_elems, ecol, ex, base);
+      else if (emode == 1) r.e = Frag<T, EW>::splat(r.c.get(0));
+      else if (emode == 2) r.e = Frag<T, EW>::splat(r.c.get(V - 1));
+      else r.e = rebuild_frag_generic<T, EW, SCHEME, RECON>(p, m, rp, ctx_of<SCHEME>(rec), ring, slot_elems, ex, base);
     } else {
       const RowCtx rc = ctx_of<SCHEME>(rec);
-      c = rebuild_frag_generic<T, V, SCHEME, RECON>(p, m, rp, rc, ring, slot_elems, xc, base);
-      e = rebuild_frag_generic<T, EW, SCHEME, RECON>(p, m, rp, rc, ring, slot_elems, ex, base);
-      if (App::NIN > 1) c2 = rebuild_frag_generic<T, V, SCHEME, RECON>(p, m, rp, rc, ring2, slot_elems, xc, base);
+      r.c = rebuild_frag_generic<T, V, SCHEME, RECON>(p, m, rp, rc, ring, slot_elems, xc, base);
+      r.e = rebuild_frag_generic<T, EW, SCHEME, RECON>(p, m, rp, rc, ring, slot_elems, ex, base);
+      if (App::NIN > 1) r.c2 = rebuild_frag_generic<T, V, SCHEME, RECON>(p, m, rp, rc, ring2, slot_elems, xc, base);
     }
-    const Frag<T, V> o = app.template row<U>(c, e, c2, lane, vy, xc, p);
+    return r;
+  };
+  // compute: the unchanged stencil on the rebuilt row (a3) and the store
+  auto compute = [&](auto uc, const Rows& r, int vy) {
+    constexpr int U = decltype(uc)::value;
+    const Frag<T, V> o = app.template row<U>(r.c, r.e, r.c2, lane, vy, xc, p);
     if (vy >= ys + VR) {  // kernel execution result -> output buffer
       if (FAST && p.vec_io) {
 #pragma unroll
@@ -114,13 +129,30 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
     }
   };
 
+#if KPERF_PIPELINE
+  // software pipeline: row vy+1 is fetched before row vy is computed
+  Rows cur = fetch(vy0);
   for (int vb = vy0; vb < vy1; vb += NWIN) {
     auto unrolled = [&](auto uc) {
       const int vy = vb + decltype(uc)::value;
-      if (vy < vy1) step(uc, vy);
+      if (vy < vy1) {
+        Rows nxt;
+        if (vy + 1 < vy1) nxt = fetch(vy + 1);
+        compute(uc, cur, vy);
+        cur = nxt;
+      }
     };
     static_for<0, NWIN>(unrolled);
   }
+#else
+  for (int vb = vy0; vb < vy1; vb += NWIN) {
+    auto unrolled = [&](auto uc) {
+      const int vy = vb + decltype(uc)::value;
+      if (vy < vy1) compute(uc, fetch(vy), vy);
+    };
+    static_for<0, NWIN>(unrolled);
+  }
+#endif
   // every copy of this item lands, then its slots go back to the producer
   const int g_end = g0 + rp.nload;
 #pragma unroll 1
@@ -154,7 +186,7 @@ __device__ __noinline__ void consumer_generic(const KParams& p, const Mask& m, c
 // Persistent CTAs: CTA b processes work items b, b + gridDim.x, ...; an item is
 // (frame, segment of seg_h output rows, strip of TW columns), strip fastest.
 template <class App, int SCHEME, int RECON, int NCW>
-__global__ void __launch_bounds__(32 * (NCW + 1), App::MINB) perf_kernel(const __grid_constant__ KParams p) {
+__global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : App::MINB) perf_kernel(const __grid_constant__ KParams p) {
   using T = typename App::T;
   constexpr int V = App::V;
   constexpr int TW = NCW * 32 * V;
