@@ -271,40 +271,59 @@ struct AppGaussSobel {
 // ---------------------------------------------------------------------------
 // K3 Median 3x3, u8: column sort of the 3-row window, then
 // med9 = med3(max of column minima, med3 of column medians, min of column maxima)
-// on packed u16x2 lanes (VIMNMX.U16x2), 2 pixels per instruction.
+// on packed 16-bit lanes, 2 pixels per instruction.  A lane holds 0x6400|v:
+// as u16 it orders like v (VIMNMX.U16x2, ALU pipe) and as fp16 it is exactly
+// 1024+v (HMNMX2), so the two instruction kinds can share the work
+// (KPERF_MEDIAN_MODE: 0 VIMNMX only, 1 HMNMX2 only, 2 alternate by word).
+#ifndef KPERF_MEDIAN_MODE
+#define KPERF_MEDIAN_MODE 2
+#endif
+template <int K>
+__device__ __forceinline__ uint32_t mn2(uint32_t a, uint32_t b) {
+  if (KPERF_MEDIAN_MODE == 1 || (KPERF_MEDIAN_MODE == 2 && (K & 1))) return hmin2u(a, b);
+  return vmin2(a, b);
+}
+template <int K>
+__device__ __forceinline__ uint32_t mx2(uint32_t a, uint32_t b) {
+  if (KPERF_MEDIAN_MODE == 1 || (KPERF_MEDIAN_MODE == 2 && (K & 1))) return hmax2u(a, b);
+  return vmax2(a, b);
+}
+
 struct AppMedian {
   using T = uint8_t;
   static constexpr int V = 16, EW = 4, VR = 1, NIN = 1, NWIN = 3, MINB = 3;
-  static constexpr int NW = V / 2 + 2;  // u16x2 words per row incl. the two halo words
+  static constexpr int NW = V / 2 + 2;  // 16-bit-pair words per row incl. the two halo words
   uint32_t r[3][NW];  // word 0 = (_, col -1), words 1..V/2 = cols 0..V-1, last = (col V, _)
   __device__ void init(const KParams&) {}
+  template <int K>
   __device__ __forceinline__ static uint32_t med3(uint32_t a, uint32_t b, uint32_t c) {
-    return vmax2(vmin2(a, b), vmin2(vmax2(a, b), c));
+    return mx2<K>(mn2<K>(a, b), mn2<K>(mx2<K>(a, b), c));
   }
   template <int U>
   __device__ __forceinline__ Frag<uint8_t, V> row(const Frag<uint8_t, V>& c, const Frag<uint8_t, EW>& e,
                                                   const Frag<uint8_t, V>&, int lane, int, int, const KParams&) {
+    constexpr uint32_t HI = 0x64646464u;  // fp16 exponent byte of 1024
     uint32_t lft = __shfl_up_sync(FULLMASK, c.w[V / 4 - 1], 1);
     uint32_t rgt = __shfl_down_sync(FULLMASK, c.w[0], 1);
     if (lane == 0) lft = e.w[0];
     if (lane == 31) rgt = e.w[0];
-    r[U][0] = __byte_perm(lft, 0, 0x4344);  // byte 3 -> high half
+    r[U][0] = __byte_perm(lft, HI, 0x4344);  // (0x6464, 0x64|col -1)
 #pragma unroll
     for (int k = 0; k < V / 4; ++k) {
-      r[U][1 + 2 * k] = __byte_perm(c.w[k], 0, 0x4140);
-      r[U][2 + 2 * k] = __byte_perm(c.w[k], 0, 0x4342);
+      r[U][1 + 2 * k] = __byte_perm(c.w[k], HI, 0x4140);
+      r[U][2 + 2 * k] = __byte_perm(c.w[k], HI, 0x4342);
     }
-    r[U][NW - 1] = __byte_perm(rgt, 0, 0x4440);  // byte 0 -> low half
+    r[U][NW - 1] = __byte_perm(rgt, HI, 0x4440);  // (0x64|col V, 0x6464)
     constexpr int A = (U + 1) % 3, B = (U + 2) % 3;
     uint32_t lo[NW], md[NW], hi[NW];
-#pragma unroll
-    for (int k = 0; k < NW; ++k) {
-      const uint32_t t1 = vmin2(r[A][k], r[B][k]), t2 = vmax2(r[A][k], r[B][k]);
-      lo[k] = vmin2(t1, r[U][k]);
-      const uint32_t t3 = vmax2(t1, r[U][k]);
-      md[k] = vmin2(t2, t3);
-      hi[k] = vmax2(t2, t3);
-    }
+    static_for<0, NW>([&](auto kc) {
+      constexpr int k = decltype(kc)::value;
+      const uint32_t t1 = mn2<k>(r[A][k], r[B][k]), t2 = mx2<k>(r[A][k], r[B][k]);
+      lo[k] = mn2<k>(t1, r[U][k]);
+      const uint32_t t3 = mx2<k>(t1, r[U][k]);
+      md[k] = mn2<k>(t2, t3);
+      hi[k] = mx2<k>(t2, t3);
+    });
     uint32_t sl[NW - 1], sm[NW - 1], sh[NW - 1];  // shifted by one column: (col 2k-1, col 2k) at [k]
 #pragma unroll
     for (int k = 0; k < NW - 1; ++k) {
@@ -313,13 +332,13 @@ struct AppMedian {
       sh[k] = __byte_perm(hi[k], hi[k + 1], 0x5432);
     }
     uint32_t out[V / 2];
-#pragma unroll
-    for (int k = 0; k < V / 2; ++k) {
-      const uint32_t mx = vmax2(vmax2(sl[k], lo[k + 1]), sl[k + 1]);
-      const uint32_t mn = vmin2(vmin2(sh[k], hi[k + 1]), sh[k + 1]);
-      const uint32_t mm = med3(sm[k], md[k + 1], sm[k + 1]);
-      out[k] = med3(mx, mm, mn);
-    }
+    static_for<0, V / 2>([&](auto kc) {
+      constexpr int k = decltype(kc)::value;
+      const uint32_t mx = mx2<k>(mx2<k>(sl[k], lo[k + 1]), sl[k + 1]);
+      const uint32_t mn = mn2<k>(mn2<k>(sh[k], hi[k + 1]), sh[k + 1]);
+      const uint32_t mm = med3<k>(sm[k], md[k + 1], sm[k + 1]);
+      out[k] = med3<k + 1>(mx, mm, mn);
+    });
     Frag<uint8_t, V> o;
 #pragma unroll
     for (int k = 0; k < V / 4; ++k) o.w[k] = __byte_perm(out[2 * k], out[2 * k + 1], 0x6420);

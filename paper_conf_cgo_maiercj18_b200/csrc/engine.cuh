@@ -51,6 +51,19 @@ struct KParams {
   float sdc, rx1, ry1, rz1, amb;  // Hotspot (Rodinia) coefficients
 };
 
+// compile-time loop: f(IC<0>{}), f(IC<1>{}), ... f(IC<N-1>{})
+template <int I>
+struct IC {
+  static constexpr int value = I;
+};
+template <int I, int N, class F>
+__device__ __forceinline__ void static_for(F&& f) {
+  if constexpr (I < N) {
+    f(IC<I>{});
+    static_for<I + 1, N>(f);
+  }
+}
+
 __device__ __forceinline__ int clampi(int v, int lo, int hi) { return v < lo ? lo : (v > hi ? hi : v); }
 
 // ---------------------------------------------------------------------------
@@ -327,8 +340,14 @@ __device__ __forceinline__ Frag<float, N> li_frag(const Frag<float, N>& a, const
                                                   int db) {
   Frag<float, N> r;
   if (da == db) {
+    if constexpr (N % 2 == 0) {  // FADD2 + FMUL2 per two samples
 #pragma unroll
-    for (int i = 0; i < N; ++i) r.v[i] = __fmul_rn(__fadd_rn(a.v[i], b.v[i]), 0.5f);
+      for (int i = 0; i < N; i += 2)
+        up2(mul2(add2(pk2(a.v[i], a.v[i + 1]), pk2(b.v[i], b.v[i + 1])), splat2(0.5f)), r.v[i], r.v[i + 1]);
+    } else {
+#pragma unroll
+      for (int i = 0; i < N; ++i) r.v[i] = __fmul_rn(__fadd_rn(a.v[i], b.v[i]), 0.5f);
+    }
   } else {
     const float fda = (float)da, fdb = (float)db, inv = __frcp_rn((float)(da + db));
 #pragma unroll

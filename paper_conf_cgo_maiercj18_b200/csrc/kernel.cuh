@@ -17,17 +17,6 @@ namespace kp {
 
 constexpr int kMaxVR = 3;  // largest vertical radius of an app (recipe table rows = seg_h + 2 VR)
 
-template <int I>
-struct IC {
-  static constexpr int value = I;
-};
-template <int I, int N, class F>
-__device__ __forceinline__ void static_for(F& f) {
-  if constexpr (I < N) {
-    f(IC<I>{});
-    static_for<I + 1, N>(f);
-  }
-}
 
 __device__ __forceinline__ void mbar_wait_u32(uint32_t addr, uint32_t parity) {
   // watchdog: a protocol bug traps (launch error) instead of hanging the GPU
@@ -51,8 +40,7 @@ __device__ __forceinline__ void mbar_arrive_u32(uint32_t addr) {
 template <class App, int SCHEME, int RECON, int NCW, bool FAST>
 __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int x0, int frame,
                                          int ys, int ye, int g0, uint32_t full_u32, uint32_t empty_u32,
-                                         const typename App::T* ring, int slot_elems, const Recipe* rtab,
-                                         int& ready, int& released) {
+                                         const typename App::T* ring, int slot_elems, const Recipe* rtab) {
   using T = typename App::T;
   constexpr int V = App::V, EW = App::EW, VR = App::VR, NWIN = App::NWIN;
   constexpr int CV = 16 / sizeof(T);  // elements of one 16-B mask-uniform chunk
@@ -72,6 +60,7 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
   T* optr = static_cast<T*>(p.out) + (long long)frame * p.out_fstride + (long long)(ys - p.out_row0) * p.W + xc;
   const int nmask = p.nr - 1;
   const int vy0 = ys - VR, vy1 = ye + VR;
+  int ready = g0 - 1, released = g0;  // this warp's ring counters (global load indices)
 
   struct Rows {  // one rebuilt input row as the lane sees it
     Frag<T, V> c, c2;
@@ -169,18 +158,16 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
 template <class App, int SCHEME, int RECON, int NCW>
 __device__ __forceinline__ void consumer_fast(const KParams& p, const Mask& m, const RowPlan& rp, int x0, int frame,
                                               int ys, int ye, int g0, uint32_t full_u32, uint32_t empty_u32,
-                                              const typename App::T* ring, int slot_elems, const Recipe* rtab,
-                                              int& ready, int& released) {
+                                              const typename App::T* ring, int slot_elems, const Recipe* rtab) {
   consumer<App, SCHEME, RECON, NCW, true>(p, m, rp, x0, frame, ys, ye, g0, full_u32, empty_u32, ring, slot_elems,
-                                          rtab, ready, released);
+                                          rtab);
 }
 template <class App, int SCHEME, int RECON, int NCW>
 __device__ __noinline__ void consumer_generic(const KParams& p, const Mask& m, const RowPlan& rp, int x0, int frame,
                                               int ys, int ye, int g0, uint32_t full_u32, uint32_t empty_u32,
-                                              const typename App::T* ring, int slot_elems, const Recipe* rtab,
-                                              int& ready, int& released) {
+                                              const typename App::T* ring, int slot_elems, const Recipe* rtab) {
   consumer<App, SCHEME, RECON, NCW, false>(p, m, rp, x0, frame, ys, ye, g0, full_u32, empty_u32, ring, slot_elems,
-                                           rtab, ready, released);
+                                           rtab);
 }
 
 // Persistent CTAs: CTA b processes work items b, b + gridDim.x, ...; an item is
@@ -220,8 +207,7 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : App:
   if (warp > nact) return;
   const uint32_t full_u32 = smem_u32(full), empty_u32 = smem_u32(empty);
 
-  int g0 = 0;  // global load index of the current item's first row
-  int ready = -1, released = 0;
+  const int g0 = 0;  // global load index of the item's first row (one item per CTA)
   {
     const int item = blockIdx.x;  // one work item per CTA (persistent variant)
     if (item >= n_items) return;
@@ -244,10 +230,10 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : App:
       const int xw = x0 + (warp - 1) * 32 * V;
       if (p.fast_ok && xw + 32 * V <= p.W)
         consumer_fast<App, SCHEME, RECON, NCW>(p, m, rp, x0, frame, ys, ye, g0, full_u32, empty_u32, ring,
-                                               slot_elems, rtab, ready, released);
+                                               slot_elems, rtab);
       else
         consumer_generic<App, SCHEME, RECON, NCW>(p, m, rp, x0, frame, ys, ye, g0, full_u32, empty_u32, ring,
-                                                  slot_elems, rtab, ready, released);
+                                                  slot_elems, rtab);
     }
   }
 }

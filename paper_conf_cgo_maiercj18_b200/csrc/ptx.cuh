@@ -70,6 +70,18 @@ __device__ __forceinline__ void st_global_v4(void* p, uint32_t a, uint32_t b, ui
                : "memory");
 }
 
+// packed fp16x2 min / max (HMNMX2).  Median lanes hold 0x6400|v (fp16 1024+v),
+// which orders the same as u16, so VIMNMX.U16x2 and HMNMX2 are interchangeable.
+__device__ __forceinline__ uint32_t hmin2u(uint32_t a, uint32_t b) {
+  uint32_t r;
+  asm("min.f16x2 %0, %1, %2;" : "=r"(r) : "r"(a), "r"(b));
+  return r;
+}
+__device__ __forceinline__ uint32_t hmax2u(uint32_t a, uint32_t b) {
+  uint32_t r;
+  asm("max.f16x2 %0, %1, %2;" : "=r"(r) : "r"(a), "r"(b));
+  return r;
+}
 // packed u16x2 min / max (VIMNMX.U16x2)
 __device__ __forceinline__ uint32_t vmin2(uint32_t a, uint32_t b) {
   uint32_t r;
