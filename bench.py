@@ -170,14 +170,21 @@ def dist_setup(args):
     ws = int(os.environ.get("WORLD_SIZE", "1"))
     rank = int(os.environ.get("RANK", "0"))
     local = int(os.environ.get("LOCAL_RANK", "0"))
+    # KPERF_BENCH_BACKEND=gloo lets several ranks share one GPU (code-path test on a
+    # 1-GPU box; NCCL refuses two ranks on one device).  Production: nccl, one GPU per rank.
+    backend = os.environ.get("KPERF_BENCH_BACKEND", "nccl")
+    dev = local % max(1, torch.cuda.device_count())
     if ws > 1:
         import torch.distributed as dist
         os.environ.setdefault("MASTER_ADDR", "127.0.0.1")
-        torch.cuda.set_device(local)
-        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+        torch.cuda.set_device(dev)
+        if backend == "nccl":
+            dist.init_process_group("nccl", device_id=torch.device("cuda", dev))
+        else:
+            dist.init_process_group(backend)
     else:
         torch.cuda.set_device(0)
-    return ws, rank, local
+    return ws, rank, dev
 
 
 def barrier(ws):
@@ -191,7 +198,8 @@ def max_over_ranks(ws, v):
         return v
     import torch
     import torch.distributed as dist
-    t = torch.tensor([v], dtype=torch.float64, device="cuda")
+    on_gpu = dist.get_backend() == "nccl"
+    t = torch.tensor([v], dtype=torch.float64, device="cuda" if on_gpu else "cpu")
     dist.all_reduce(t, op=dist.ReduceOp.MAX)
     return float(t.item())
 
@@ -352,6 +360,17 @@ def main():
         achieved = algo_b / (ms * 1e-3) / 1e9
         kkey = f"{app}{cfg['r']}_{cfg['scheme']}_{cfg['rate'][0]}-{cfg['rate'][1]}_{cfg['recon']}"
         tr = ncu_traffic(kkey)
+        alu = None
+        if u8:  # the median is ALU-pipe bound: roofline on ALU lane-ops
+            # sorted-column network on 16-bit pairs, per 2 output pixels: column sort 6,
+            # combine 12 min/max, 3 one-column shifts + 1 unpack + 0.5 pack PRMT = 22.5 lane-ops
+            ops_px = 22.5 / 2
+            sm_mhz = 1965.0
+            alu_peak = 148 * 4 * 16 * sm_mhz * 1e6 / 1e12  # T lane-ops/s: 0.5 warp-inst/clk/SMSP
+            alu_ach = ops_px * px_step / (ms * 1e-3) / 1e12
+            alu = {"bound": "alu", "achieved": alu_ach, "peak": alu_peak, "unit": "Tlane-op/s",
+                   "frac": alu_ach / alu_peak, "ops_per_px": ops_px,
+                   "peak_derivation": "148 SM x 4 SMSP x 16 lanes/clk (ALU pipe, 1 warp-inst / 2 clk) x 1965 MHz"}
         pmix = mixed_peak_gbs(x.data_ptr(), yex.data_ptr(), px_step * es, cfg["scheme"], cfg["rate"], G,
                               stream=stream.cuda_stream) if not u8 else None
         result = {
@@ -374,6 +393,9 @@ def main():
             "clocks": clk.summary(),
             "gpu_launches": args.steps,
         }
+        if alu:
+            result["roofline_hbm"] = result["roofline"]
+            result["roofline"] = alu
         # e2e through the C ABI with pinned host buffers (one frame per step)
         result["e2e"] = bench_e2e(kp, cfg, stream, args, ws, x)
         if not args.no_variants and args.config == "C2":
@@ -472,7 +494,7 @@ def bench_hotspot(args, cfg, ws, rank, local, stream, peak, peak_src):
     if ws > 1:
         import torch.distributed as dist
         uid = kp.perf_comm_unique_id() if rank == 0 else bytes(128)
-        t = torch.tensor(list(uid), dtype=torch.uint8, device="cuda")
+        t = torch.tensor(list(uid), dtype=torch.uint8, device="cuda" if dist.get_backend() == "nccl" else "cpu")
         dist.broadcast(t, 0)
         uid = bytes(t.cpu().tolist())
         kp.perf_comm_init(plan.handle, uid, rank, ws)

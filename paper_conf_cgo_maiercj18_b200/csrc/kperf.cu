@@ -79,7 +79,8 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
                                KParams& k, unsigned& grid, size_t& smem) {
   const int es = (int)elem_size(P->app);
   const int CV = 16 / es;  // elements per 16-B chunk (load / store / alignment unit)
-  const int V = P->app == PERF_APP_MEDIAN ? 16 : 8;  // elements per consumer lane per row (apps.cuh)
+  // elements per consumer lane per row (must match App::V in apps.cuh)
+  const int V = P->app == PERF_APP_MEDIAN ? 16 : 8;
   const int NCW = kp::kNCW;
   const int TW = NCW * 32 * V;
   const int Hg = P->global_h > 0 ? (int)P->global_h : P->H;
