@@ -23,14 +23,14 @@ _HERE = os.path.dirname(os.path.abspath(__file__))
 _LIB_PATH = os.path.join(_HERE, "liboracle.so")
 
 APPS = {"gaussian": 0, "sobel": 1, "median": 2, "hotspot": 3, "gauss_sobel": 4, "inversion": 5}
-SCHEMES = {"none": 0, "row": 1, "col": 2, "checker": 3}
+SCHEMES = {"none": 0, "row": 1, "col": 2, "checker": 3, "stencil1": 4}
 RECONS = {"nn": 0, "li": 1}
 METRICS = {"mre": 0, "me": 1, "mae": 2}
 
 
 class OrcParams(ctypes.Structure):
     _fields_ = [(n, ctypes.c_int) for n in
-                ("app", "W", "H", "radius", "scheme", "num", "den", "recon", "granule")]
+                ("app", "W", "H", "radius", "scheme", "num", "den", "recon", "granule", "tile_w", "tile_h")]
 
 
 def build(force: bool = False) -> str:
@@ -81,9 +81,9 @@ def lib():
     return _lib
 
 
-def params(app="gaussian", W=0, H=0, radius=2, scheme="none", rate=(0, 1), recon="nn", granule=8):
+def params(app="gaussian", W=0, H=0, radius=2, scheme="none", rate=(0, 1), recon="nn", granule=8, tile=(16, 16)):
     num, den = rate
-    return OrcParams(APPS[app], W, H, radius, SCHEMES[scheme], num, den, RECONS[recon], granule)
+    return OrcParams(APPS[app], W, H, radius, SCHEMES[scheme], num, den, RECONS[recon], granule, tile[0], tile[1])
 
 
 def _ptr(a: np.ndarray):

@@ -25,7 +25,7 @@
  * coordinates, line 0 kept), R3 (column/checker cells are G pixels wide),
  * R4 (checkerboard lattice q = (x/G + y) mod den).                          */
 int orc_is_kept(const orc_params* p, int x, int y) {
-  if (p->scheme == ORC_NONE || p->num == 0) return 1;
+  if (p->scheme == ORC_NONE || p->scheme == ORC_STENCIL1 || p->num == 0) return 1;
   const int den = p->den;
   int q;
   if (p->scheme == ORC_ROW) q = y % den;
@@ -135,6 +135,16 @@ void orc_reconstruct_u8(const orc_params* p, const uint8_t* img, uint8_t* R) {
 }
 
 /* ------------------------------------------------------------------------ */
+/* Stencil1 (PAPER.md:479-490, Fig. 5; :819-821 "Stencil1 is perforation of
+ * the boundaries of a work group tile and uses nearest-neighbor
+ * interpolation"): a work group fetches only its tile's interior; the halo
+ * elements its stencil reads are rebuilt by NN from the loaded tile, i.e. the
+ * tile-border element (reading R18).  The stencil of output (x, y) therefore
+ * reads the input at coordinates clamped to its own tile (and to the image).
+ * LI needs loaded elements on both sides, which a halo element never has, so
+ * it falls back to NN. */
+static int tile_lo(int v, int t) { return (v / t) * t; }
+
 /* Step 3: the unchanged application stencils (Sec. 6.1).
  * Reading R8: clamp-to-edge addressing at image borders.  R9: Gaussian
  * weights are binomial b(x)b(y) / (sum b)^2, b = [1,2,1] (r=1) or
@@ -181,8 +191,28 @@ static int median9(int* v) {
   return v[4];
 }
 
+static void run_stencil1_f32(const orc_params* p, const float* in, double* out) {
+  const int W = p->W, H = p->H, r = (p->app == ORC_INVERSION) ? 0 : p->radius;
+  const int n = 2 * r + 1;
+  double win[25];
+  for (int y = 0; y < H; ++y)
+    for (int x = 0; x < W; ++x) {
+      const int tx0 = tile_lo(x, p->tile_w), ty0 = tile_lo(y, p->tile_h);
+      const int tx1 = (tx0 + p->tile_w < W ? tx0 + p->tile_w : W) - 1;
+      const int ty1 = (ty0 + p->tile_h < H ? ty0 + p->tile_h : H) - 1;
+      for (int i = -r; i <= r; ++i)
+        for (int j = -r; j <= r; ++j)
+          win[(i + r) * n + (j + r)] = (double)in[(long long)clampi(y + i, ty0, ty1) * W + clampi(x + j, tx0, tx1)];
+      out[(long long)y * W + x] = stencil_f(p->app, r, win, n, n, r, r);
+    }
+}
+
 void orc_run_f32(const orc_params* p, const float* in, double* out) {
   const int W = p->W, H = p->H;
+  if (p->scheme == ORC_STENCIL1 && (p->app == ORC_GAUSSIAN || p->app == ORC_SOBEL || p->app == ORC_INVERSION)) {
+    run_stencil1_f32(p, in, out);
+    return;
+  }
   const long long n = (long long)W * H;
   double* R = (double*)malloc(sizeof(double) * n);
   orc_reconstruct_f32(p, in, R);
@@ -202,6 +232,19 @@ void orc_run_f32(const orc_params* p, const float* in, double* out) {
 
 void orc_run_u8(const orc_params* p, const uint8_t* in, uint8_t* out) {
   const int W = p->W, H = p->H;
+  if (p->scheme == ORC_STENCIL1) {
+    for (int y = 0; y < H; ++y)
+      for (int x = 0; x < W; ++x) {
+        const int tx0 = tile_lo(x, p->tile_w), ty0 = tile_lo(y, p->tile_h);
+        const int tx1 = (tx0 + p->tile_w < W ? tx0 + p->tile_w : W) - 1;
+        const int ty1 = (ty0 + p->tile_h < H ? ty0 + p->tile_h : H) - 1;
+        int v[9], k = 0;
+        for (int i = -1; i <= 1; ++i)
+          for (int j = -1; j <= 1; ++j) v[k++] = in[(long long)clampi(y + i, ty0, ty1) * W + clampi(x + j, tx0, tx1)];
+        out[(long long)y * W + x] = (uint8_t)median9(v);
+      }
+    return;
+  }
   uint8_t* R = (uint8_t*)malloc((size_t)W * H);
   orc_reconstruct_u8(p, in, R);
   for (int y = 0; y < H; ++y)
@@ -218,6 +261,17 @@ void orc_run_u8(const orc_params* p, const uint8_t* in, uint8_t* out) {
 /* One output pixel: rebuild just the window it reads (same definitions). */
 double orc_run_pixel_f32(const orc_params* p, const float* in, int x, int y) {
   const int W = p->W, H = p->H;
+  if (p->scheme == ORC_STENCIL1) {
+    const int r = (p->app == ORC_INVERSION) ? 0 : p->radius, n = 2 * r + 1;
+    const int tx0 = tile_lo(x, p->tile_w), ty0 = tile_lo(y, p->tile_h);
+    const int tx1 = (tx0 + p->tile_w < W ? tx0 + p->tile_w : W) - 1;
+    const int ty1 = (ty0 + p->tile_h < H ? ty0 + p->tile_h : H) - 1;
+    double win[25];
+    for (int i = -r; i <= r; ++i)
+      for (int j = -r; j <= r; ++j)
+        win[(i + r) * n + (j + r)] = (double)in[(long long)clampi(y + i, ty0, ty1) * W + clampi(x + j, tx0, tx1)];
+    return stencil_f(p->app, r, win, n, n, r, r);
+  }
   if (p->app == ORC_GAUSS_SOBEL) {
     /* Gaussian5 at the 3x3 clamped neighbours, each from a 5x5 rebuilt window */
     double g[9];
@@ -251,6 +305,14 @@ double orc_run_pixel_f32(const orc_params* p, const float* in, int x, int y) {
 
 int orc_run_pixel_u8(const orc_params* p, const uint8_t* in, int x, int y) {
   int v[9], k = 0;
+  if (p->scheme == ORC_STENCIL1) {
+    const int tx0 = tile_lo(x, p->tile_w), ty0 = tile_lo(y, p->tile_h);
+    const int tx1 = (tx0 + p->tile_w < p->W ? tx0 + p->tile_w : p->W) - 1;
+    const int ty1 = (ty0 + p->tile_h < p->H ? ty0 + p->tile_h : p->H) - 1;
+    for (int i = -1; i <= 1; ++i)
+      for (int j = -1; j <= 1; ++j) v[k++] = in[(long long)clampi(y + i, ty0, ty1) * p->W + clampi(x + j, tx0, tx1)];
+    return median9(v);
+  }
   for (int i = -1; i <= 1; ++i)
     for (int j = -1; j <= 1; ++j)
       v[k++] = orc_R_u8(p, in, clampi(x + j, 0, p->W - 1), clampi(y + i, 0, p->H - 1));

@@ -24,7 +24,7 @@ extern "C" {
 
 enum { ORC_GAUSSIAN = 0, ORC_SOBEL = 1, ORC_MEDIAN = 2, ORC_HOTSPOT = 3, ORC_GAUSS_SOBEL = 4,
        ORC_INVERSION = 5 };
-enum { ORC_NONE = 0, ORC_ROW = 1, ORC_COL = 2, ORC_CHECKER = 3 };
+enum { ORC_NONE = 0, ORC_ROW = 1, ORC_COL = 2, ORC_CHECKER = 3, ORC_STENCIL1 = 4 };
 enum { ORC_NN = 0, ORC_LI = 1 };
 enum { ORC_METRIC_MRE = 0, ORC_METRIC_ME = 1, ORC_METRIC_MAE = 2 };
 
@@ -33,6 +33,7 @@ typedef struct {
   int scheme, num, den; /* skipped fraction num/den; num in {0, 1, den-1} */
   int recon;
   int granule;          /* G: pixels per column/checker cell (>= 1) */
+  int tile_w, tile_h;   /* STENCIL1: work-group tile of output pixels */
 } orc_params;
 
 /* Step 1 -- perforation mask (1 = loaded / kept, 0 = skipped). */

@@ -430,3 +430,74 @@ def test_p12_synth_ranges():
     T, Pw = synth.hotspot(5, 64, 48)
     assert np.all(T * 64 == np.round(T * 64)) and T.min() > 300 and T.max() < 340
     assert Pw.min() >= 0 and np.all(Pw * 131072 == np.round(Pw * 131072))
+
+
+# --------------------------------------------------------------------------
+# P13: Stencil1 (PAPER.md:479-490, Fig. 5; :819-821) -- the tile fetches only
+# its interior, the halo is rebuilt by NN from the tile border
+def _np_stencil1(app, r, img, tw, th):
+    """independent formulation: pad every tile with its own border, filter it"""
+    H, W = img.shape
+    out = np.zeros((H, W))
+    for ty in range(0, H, th):
+        for tx in range(0, W, tw):
+            t = img[ty:ty + th, tx:tx + tw]
+            if app == "median":
+                out[ty:ty + th, tx:tx + tw] = _np_median(t)
+            else:
+                sob, gau = _np_sobel(t, r)
+                out[ty:ty + th, tx:tx + tw] = sob if app == "sobel" else gau
+    return out
+
+
+@pytest.mark.parametrize("app,r", [("gaussian", 1), ("gaussian", 2), ("sobel", 1), ("sobel", 2), ("median", 1)])
+@pytest.mark.parametrize("tile", [(16, 16), (32, 8), (8, 4), (5, 7)])
+def test_p13_stencil1_per_tile(app, r, tile):
+    W, H = 53, 41
+    img = synth.image("natural", 13, W, H, np.uint8 if app == "median" else np.float32)
+    p = P(app, W, H, r, "stencil1", (0, 1), "nn")
+    p.tile_w, p.tile_h = tile
+    got = oracle.run(p, img)
+    want = _np_stencil1(app, r, img, *tile)
+    if app == "median":
+        assert np.array_equal(got, want)
+    else:
+        assert np.allclose(got, want, rtol=1e-13, atol=1e-9)
+    xs, ys = np.arange(0, W, 3), np.arange(0, H, 3)[: len(np.arange(0, W, 3))]
+    xs = xs[: len(ys)]
+    assert np.array_equal(oracle.run_pixels(p, img, xs, ys), got[ys, xs])
+
+
+def test_p13_stencil1_invariants():
+    W, H = 40, 30
+    img = synth.image("natural", 14, W, H)
+    p = P("gaussian", W, H, 2, "stencil1")
+    p.tile_w, p.tile_h = 64, 64  # one tile covers the image: exact
+    assert np.array_equal(oracle.run(p, img), oracle.run(P("gaussian", W, H, 2), img))
+    c = np.full((H, W), 61.0, dtype=np.float32)
+    p.tile_w, p.tile_h = 8, 8
+    assert np.all(oracle.run(p, c) == 61.0)
+    ps = P("sobel", W, H, 1, "stencil1")
+    ps.tile_w, ps.tile_h = 8, 8
+    assert np.all(oracle.run(ps, c) == 0.0)
+    # interior pixels of a tile (>= r from its border) are exact
+    ex = oracle.run(P("gaussian", W, H, 2), img)
+    st = oracle.run(p, img)
+    inner = np.zeros((H, W), bool)
+    for ty in range(0, H, 8):
+        for tx in range(0, W, 8):
+            inner[ty + 2:min(ty + 6, H - 2), tx + 2:min(tx + 6, W - 2)] = True
+    assert np.array_equal(st[inner], ex[inner]) and not np.array_equal(st, ex)
+
+
+def test_p13_stencil1_paper_claims():
+    """'The error for Stencil1 is very low and always less than 1%' and below
+    Rows1:NN, on a natural-image stand-in"""
+    W = H = 256
+    img = synth.image("natural", synth.SEED_C2 + 1, W, H)
+    ex = oracle.run(P("gaussian", W, H, 1), img)
+    p = P("gaussian", W, H, 1, "stencil1")
+    p.tile_w, p.tile_h = 16, 16
+    e_s1 = oracle.error("mre", ex, oracle.run(p, img))[0]
+    e_r1 = oracle.error("mre", ex, oracle.run(P("gaussian", W, H, 1, "row", (1, 2), "nn"), img))[0]
+    assert e_s1 < 0.01 and e_s1 < e_r1
