@@ -469,6 +469,15 @@ def bench_variants(kp, cfg, x, y, yex, stream, peak, ws):
                                 "mix_ceiling": (pm / bytes_per_px(app, scheme, rate)) / (pm_ex / 8.0)
                                 if pm and pm_ex else None})
                     p.close()
+        for tile in ((16, 16), (32, 8)):  # NEXT-1: the paper's Stencil1 (halo-only perforation)
+            p = kp.Plan(app, W, H, r, "stencil1", (0, 1), "nn", batch=B, tile1_w=tile[0], tile1_h=tile[1])
+            ms = time_kernel(lambda: p.run(x, y, stream), stream, 10, 3)
+            err, _ = p.error(yex, y, stream)
+            out.append({"app": app, "r": r, "scheme": "stencil1", "tile": list(tile), "rate": [0, 1], "recon": "nn",
+                        "ms": ms, "mpixel_s": px / ms / 1e3, "speedup": ms_ex / ms, "error": err,
+                        "hbm_gbs": 8 * px / ms / 1e6, "frac": 8 * px / ms / 1e6 / peak,
+                        "frac_mix": 8 * px / ms / 1e6 / pm_ex if pm_ex else None})
+            p.close()
         ex.close()
     return out
 

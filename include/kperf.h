@@ -57,7 +57,11 @@ typedef enum {
   PERF_SCHEME_NONE = 0,    /* exact kernel: every input element is loaded */
   PERF_SCHEME_ROW = 1,     /* skip whole rows; rebuilt along y */
   PERF_SCHEME_COL = 2,     /* skip G-pixel column granules; rebuilt along x */
-  PERF_SCHEME_CHECKER = 3  /* skip G-pixel cells on a diagonal lattice; rebuilt along y */
+  PERF_SCHEME_CHECKER = 3, /* skip G-pixel cells on a diagonal lattice; rebuilt along y */
+  PERF_SCHEME_STENCIL1 = 4 /* the paper's Stencil1 (Sec. 4.4, Fig. 5): a work-group tile of
+                              TILE1_W x TILE1_H outputs loads only its interior; its halo is
+                              rebuilt by NN from the tile border.  rate must be {0, 1}.
+                              Gaussian, Sobel, Median, Inversion. */
 } perf_scheme;
 
 /* Reconstruction techniques (Sec. 5.1). */
@@ -95,7 +99,9 @@ enum {
   PERF_KEY_METRIC = 8,         /* perf_metric used by perf_error (default: MRE; ME for Sobel apps) */
   PERF_KEY_LOADER = 9,         /* 0 auto, 1 TMA bulk rows, 2 cp.async 16 B, 3 scalar (any alignment) */
   PERF_KEY_RING = 10,          /* shared-memory ring depth in rows (0 = auto) */
-  PERF_KEY_HALO_ROWS = 11      /* read-only: rows a Hotspot band exchanges with each neighbour per step */
+  PERF_KEY_HALO_ROWS = 11,     /* read-only: rows a Hotspot band exchanges with each neighbour per step */
+  PERF_KEY_TILE1_W = 12,       /* STENCIL1 tile width: power of two, 16..256 (fp32) / 16..512 (u8); default 16 */
+  PERF_KEY_TILE1_H = 13        /* STENCIL1 tile height, 1..1024; default 16 */
 };
 
 /* Create a plan.  Validates: W, H >= 1; radius allowed for the app (Gaussian,

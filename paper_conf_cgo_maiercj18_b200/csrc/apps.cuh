@@ -18,8 +18,10 @@ namespace kp {
 constexpr unsigned FULLMASK = 0xFFFFFFFFu;
 
 // x[0 .. V+2RH): samples at columns xc-RH .. xc+V-1+RH of the rebuilt row
+// hf: bit 0 / bit 1 = the lane's left / right edge is a Stencil1 tile border:
+// the halo there is rebuilt by NN from the tile (the lane's own edge sample).
 template <int RH, int EW, int V>
-__device__ __forceinline__ void ext_row(const Frag<float, V>& c, const Frag<float, EW>& e, int lane,
+__device__ __forceinline__ void ext_row(const Frag<float, V>& c, const Frag<float, EW>& e, int lane, uint32_t hf,
                                         float (&x)[V + 2 * RH]) {
   static_assert(RH <= EW, "edge fragment too small");
 #pragma unroll
@@ -30,6 +32,8 @@ __device__ __forceinline__ void ext_row(const Frag<float, V>& c, const Frag<floa
     float r = __shfl_down_sync(FULLMASK, c.v[k - 1], 1);
     if (lane == 0) l = e.v[EW - k];
     if (lane == 31) r = e.v[k - 1];
+    if (hf & 1u) l = c.v[0];
+    if (hf & 2u) r = c.v[V - 1];
     x[RH - k] = l;
     x[RH + V - 1 + k] = r;
   }
@@ -56,9 +60,9 @@ struct AppGauss {  // K1 Gaussian, binomial (2R+1)^2, fp32
   __device__ void init(const KParams&) {}
   template <int U>
   __device__ __forceinline__ Frag<float, V> row(const Frag<float, V>& c, const Frag<float, EW>& e,
-                                                const Frag<float, V>&, int lane, int, int, const KParams&) {
+                                                const Frag<float, V>&, int lane, uint32_t hf, int, int, const KParams&) {
     float x[V + 2 * R];
-    ext_row<R, EW, V>(c, e, lane, x);
+    ext_row<R, EW, V>(c, e, lane, hf, x);
 #pragma unroll
     for (int j = 0; j < V / 2; ++j) h[U][j] = pk2(smooth<R>(x + 2 * j), smooth<R>(x + 2 * j + 1));
     const f2 scale = splat2(R == 1 ? 1.f / 16.f : 1.f / 256.f);
@@ -85,9 +89,9 @@ struct AppSobel {  // K5 Sobel, |(Gx, Gy)|, fp32
   __device__ void init(const KParams&) {}
   template <int U>
   __device__ __forceinline__ Frag<float, V> row(const Frag<float, V>& c, const Frag<float, EW>& e,
-                                                const Frag<float, V>&, int lane, int, int, const KParams&) {
+                                                const Frag<float, V>&, int lane, uint32_t hf, int, int, const KParams&) {
     float x[V + 2 * R];
-    ext_row<R, EW, V>(c, e, lane, x);
+    ext_row<R, EW, V>(c, e, lane, hf, x);
 #pragma unroll
     for (int j = 0; j < V / 2; ++j) {
       sx[U][j] = pk2(smooth<R>(x + 2 * j), smooth<R>(x + 2 * j + 1));
@@ -125,7 +129,7 @@ struct AppInversion {  // K2 Inversion, 255 - x
   __device__ void init(const KParams&) {}
   template <int U>
   __device__ __forceinline__ Frag<float, V> row(const Frag<float, V>& c, const Frag<float, EW>&,
-                                                const Frag<float, V>&, int, int, int, const KParams&) {
+                                                const Frag<float, V>&, int, uint32_t, int, int, const KParams&) {
     Frag<float, V> o;
 #pragma unroll
     for (int i = 0; i < V; ++i) o.v[i] = 255.f - c.v[i];
@@ -149,9 +153,9 @@ struct AppHotspot {
   }
   template <int U>
   __device__ __forceinline__ Frag<float, V> row(const Frag<float, V>& c, const Frag<float, EW>& e,
-                                                const Frag<float, V>& c2, int lane, int, int, const KParams&) {
+                                                const Frag<float, V>& c2, int lane, uint32_t, int, int, const KParams&) {
     float x[V + 2];
-    ext_row<1, EW, V>(c, e, lane, x);
+    ext_row<1, EW, V>(c, e, lane, 0u, x);
 #pragma unroll
     for (int i = 0; i < V; ++i) {
       tc[U][i] = x[i + 1];
@@ -191,10 +195,10 @@ struct AppGaussSobel {
   }
   template <int U>
   __device__ __forceinline__ Frag<float, V> row(const Frag<float, V>& c, const Frag<float, EW>& e,
-                                                const Frag<float, V>&, int lane, int vy, int xc,
+                                                const Frag<float, V>&, int lane, uint32_t, int vy, int xc,
                                                 const KParams& p) {
     float x[V + 4];  // columns xc-2 .. xc+V+1
-    ext_row<2, EW, V>(c, e, lane, x);
+    ext_row<2, EW, V>(c, e, lane, 0u, x);
     // edge column (lane 0: xc-1 from e = cols xc-4..xc-1; lane 31: xc+V from e = cols xc+V..xc+V+3)
     float he;
     if (lane < 16) {
@@ -301,12 +305,15 @@ struct AppMedian {
   }
   template <int U>
   __device__ __forceinline__ Frag<uint8_t, V> row(const Frag<uint8_t, V>& c, const Frag<uint8_t, EW>& e,
-                                                  const Frag<uint8_t, V>&, int lane, int, int, const KParams&) {
+                                                  const Frag<uint8_t, V>&, int lane, uint32_t hf, int, int,
+                                                  const KParams&) {
     constexpr uint32_t HI = 0x64646464u;  // fp16 exponent byte of 1024
     uint32_t lft = __shfl_up_sync(FULLMASK, c.w[V / 4 - 1], 1);
     uint32_t rgt = __shfl_down_sync(FULLMASK, c.w[0], 1);
     if (lane == 0) lft = e.w[0];
     if (lane == 31) rgt = e.w[0];
+    if (hf & 1u) lft = c.w[0] << 24;           // Stencil1 tile border: col -1 := col 0
+    if (hf & 2u) rgt = c.w[V / 4 - 1] >> 24;  // col V := col V-1
     r[U][0] = __byte_perm(lft, HI, 0x4344);  // (0x6464, 0x64|col -1)
 #pragma unroll
     for (int k = 0; k < V / 4; ++k) {

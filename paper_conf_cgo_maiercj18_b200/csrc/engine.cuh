@@ -27,7 +27,7 @@
 
 namespace kp {
 
-enum { S_NONE = 0, S_ROW = 1, S_COL = 2, S_CHECKER = 3 };
+enum { S_NONE = 0, S_ROW = 1, S_COL = 2, S_CHECKER = 3, S_STENCIL1 = 4 };
 enum { R_NN = 0, R_LI = 1 };
 enum { L_AUTO = 0, L_BULK = 1, L_ASYNC16 = 2, L_SCALAR = 3 };
 
@@ -48,6 +48,7 @@ struct KParams {
   int row_elems;             // TW + 2*hx
   int fast_ok;               // every V-chunk lies in one mask cell (G % V == 0 or row scheme)
   int vec_io;                // W % V == 0 and 16-B aligned buffers
+  int tile1_w, tile1_h;      // Stencil1 work-group tile
   float sdc, rx1, ry1, rz1, amb;  // Hotspot (Rodinia) coefficients
 };
 
@@ -159,7 +160,7 @@ struct Mask {
 
 template <int SCHEME>
 __device__ __forceinline__ bool px_kept(const KParams& p, const Mask& m, int x, int y) {
-  if (SCHEME == S_NONE) return true;
+  if (SCHEME == S_NONE || SCHEME == S_STENCIL1) return true;
   if (SCHEME == S_ROW) return m.phase_kept(y % m.den);
   if (SCHEME == S_COL) return m.phase_kept((x / p.G) % m.den);
   return m.phase_kept((x / p.G + y) % m.den);
@@ -175,8 +176,9 @@ __device__ __forceinline__ RowPlan make_row_plan(const KParams& p, const Mask& m
   RowPlan r;
   r.lim_lo = max(0, p.avail0);
   r.lim_hi = min(p.Hg, p.avail1) - 1;
-  const int ya = clampi(ys - VR, r.lim_lo, r.lim_hi);
-  const int yb = clampi(ye - 1 + VR, r.lim_lo, r.lim_hi);
+  const int vr = SCHEME == S_STENCIL1 ? 0 : VR;  // Stencil1: the tile's own rows only
+  const int ya = clampi(ys - vr, r.lim_lo, r.lim_hi);
+  const int yb = clampi(ye - 1 + vr, r.lim_lo, r.lim_hi);
   if (SCHEME == S_ROW) {
     const int ta = ya % m.den, tb = yb % m.den;
     r.lo = m.phase_kept(ta) ? ya : ya - m.dlo(ta);
@@ -378,7 +380,8 @@ __device__ __forceinline__ uint8_t li_px(uint8_t a, uint8_t b, int da, int db) {
 
 // A row recipe: everything a consumer needs to rebuild one virtual input row,
 // computed once per CTA into shared memory.
-//   y     clamped global row;  need = need_hi | need_lo << 16 (ring indices)
+//   y     clamped global row;  need = need_hi | emit << 15 | need_lo << 16 (ring
+//         indices; emit: this row completes an output row)
 //   info  slot_a | slot_b << 8 | ym << 16 | da << 20 | db << 24 | kept << 28 |
 //         li << 29 | has_a << 30 | has_b << 31
 //   wa    LI weight of the lower sample: value = b + (a - b) * wa, wa = db/(da+db)
@@ -399,10 +402,32 @@ __device__ __forceinline__ bool rc_li(uint32_t i) { return (i >> 29) & 1; }
 __device__ __forceinline__ bool rc_has_a(uint32_t i) { return (i >> 30) & 1; }
 __device__ __forceinline__ bool rc_has_b(uint32_t i) { return (i >> 31) & 1; }
 
+// number of virtual input rows (recipes) of a segment
+template <int SCHEME>
+__device__ __forceinline__ int n_recipes(const KParams& p, int ys, int ye, int VR) {
+  if (SCHEME != S_STENCIL1) return ye - ys + 2 * VR;
+  const int th = p.tile1_h, nt = (ye - ys + th - 1) / th;
+  return (nt - 1) * (th + 2 * VR) + (ye - (ys + (nt - 1) * th)) + 2 * VR;
+}
+
+// virtual row i of a segment -> (row to rebuild, emits an output row?)
+template <int SCHEME>
+__device__ __forceinline__ int virtual_row(const KParams& p, const RowPlan& rp, int ys, int ye, int VR, int i,
+                                           int& emit) {
+  if (SCHEME != S_STENCIL1) {
+    emit = i >= 2 * VR;
+    return clampi(ys - VR + i, rp.lim_lo, rp.lim_hi);
+  }
+  // Stencil1: each tile of tile1_h rows is its own clamped window (Fig. 5)
+  const int th = p.tile1_h, per = th + 2 * VR, t = i / per, k = i - t * per;
+  const int ty0 = ys + t * th, ty1 = min(ty0 + th, ye);
+  emit = k >= 2 * VR;
+  return clampi(ty0 - VR + k, ty0, ty1 - 1);
+}
+
 template <int SCHEME, int RECON>
-__device__ __forceinline__ Recipe make_recipe(const KParams& p, const Mask& m, const RowPlan& rp, int vy) {
+__device__ __forceinline__ Recipe make_recipe(const KParams& p, const Mask& m, const RowPlan& rp, int y, int emit) {
   Recipe r;
-  const int y = clampi(vy, rp.lim_lo, rp.lim_hi);
   const int ym = y % m.den, nmask = p.nr - 1;
   int need_hi, need_lo, sa = 0, sb = 0, da = 1, db = 1, kept = 1, li = 0, ha = 0, hb = 0;
   float wa = 1.f;
@@ -440,7 +465,7 @@ __device__ __forceinline__ Recipe make_recipe(const KParams& p, const Mask& m, c
     need_hi = need_lo = y - rp.lo;
   }
   r.y = y;
-  r.need = need_hi | (need_lo << 16);
+  r.need = need_hi | (emit << 15) | (need_lo << 16);
   r.info = (uint32_t)sa | ((uint32_t)sb << 8) | ((uint32_t)ym << 16) | ((uint32_t)da << 20) |
            ((uint32_t)db << 24) | ((uint32_t)kept << 28) | ((uint32_t)li << 29) | ((uint32_t)ha << 30) |
            ((uint32_t)hb << 31);
@@ -528,7 +553,7 @@ __device__ __forceinline__ Frag<T, N> rebuild_frag(const KParams& p, const Mask&
                                                    const Recipe& rec, const ChunkInfo& ci, const T* ring,
                                                    int slot_elems, int col, int fx, int base) {
   const uint32_t info = rec.info;
-  if (SCHEME == S_NONE) return ldf<T, N>(ring + rc_slot_a(info) * slot_elems + col);
+  if (SCHEME == S_NONE || SCHEME == S_STENCIL1) return ldf<T, N>(ring + rc_slot_a(info) * slot_elems + col);
   if (SCHEME == S_ROW) {
     if (RECON == R_NN || rc_kept(info)) return ldf<T, N>(ring + rc_slot_a(info) * slot_elems + col);
     const Frag<T, N> a = ldf<T, N>(ring + rc_slot_a(info) * slot_elems + col);
@@ -598,7 +623,7 @@ template <typename T, int SCHEME, int RECON>
 __device__ __noinline__ T rebuild_px(const KParams& p, const Mask& m, const RowPlan& rp, const RowCtx& rc,
                                      const T* ring, int slot_elems, int base, int x) {
   const int col = x - base;
-  if (SCHEME == S_NONE) return ring[rc.slot_c * slot_elems + col];
+  if (SCHEME == S_NONE || SCHEME == S_STENCIL1) return ring[rc.slot_c * slot_elems + col];
   if (SCHEME == S_ROW) {
     if (rc.kept) return ring[rc.slot_c * slot_elems + col];
     // (an NN-rebuilt row is marked kept with slot_a = the chosen loaded row)

@@ -55,22 +55,29 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
   const int emode = (ex >= 0 && ex + EW <= p.W) ? 0 : (ex < 0 ? 1 : (ex == p.W ? 2 : 3));
   const int ccol = xc - base, ecol = ex - base;
   const T* ring2 = ring + p.row_elems;  // second input (Hotspot power)
+  // Stencil1: lane edges that are tile borders take their halo from the tile itself
+  const uint32_t hf = SCHEME == S_STENCIL1
+                          ? (uint32_t)((xc % p.tile1_w) == 0) | ((uint32_t)(((xc + V) % p.tile1_w) == 0) << 1)
+                          : 0u;
   App app;
   app.init(p);
   T* optr = static_cast<T*>(p.out) + (long long)frame * p.out_fstride + (long long)(ys - p.out_row0) * p.W + xc;
   const int nmask = p.nr - 1;
-  const int vy0 = ys - VR, vy1 = ye + VR;
+  const int vy0 = ys - VR;
+  const int nv = n_recipes<SCHEME>(p, ys, ye, VR);  // virtual input rows of this segment
   int ready = g0 - 1, released = g0;  // this warp's ring counters (global load indices)
 
   struct Rows {  // one rebuilt input row as the lane sees it
     Frag<T, V> c, c2;
     Frag<T, EW> e;
+    int emit;
   };
   // fetch: recipe, ring release/wait, rebuild from shared memory (a1/a2)
-  auto fetch = [&](int vy) {
+  auto fetch = [&](int i) {
     Rows r;
-    const Recipe rec = rtab[vy - vy0];
-    const int need_hi = g0 + (rec.need & 0xFFFF), need_lo = g0 + (int)((uint32_t)rec.need >> 16);
+    const Recipe rec = rtab[i];
+    const int need_hi = g0 + (rec.need & 0x7FFF), need_lo = g0 + (int)((uint32_t)rec.need >> 16);
+    r.emit = (rec.need >> 15) & 1;
     // release ring slots no later row reads (earlier rows are already in registers)
 #pragma unroll 1
     while (released < need_lo) {
@@ -101,8 +108,8 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
   // compute: the unchanged stencil on the rebuilt row (a3) and the store
   auto compute = [&](auto uc, const Rows& r, int vy) {
     constexpr int U = decltype(uc)::value;
-    const Frag<T, V> o = app.template row<U>(r.c, r.e, r.c2, lane, vy, xc, p);
-    if (vy >= ys + VR) {  // kernel execution result -> output buffer
+    const Frag<T, V> o = app.template row<U>(r.c, r.e, r.c2, lane, hf, vy, xc, p);
+    if (r.emit) {  // kernel execution result -> output buffer (output rows in order)
       if (FAST && p.vec_io) {
 #pragma unroll
         for (int q = 0; q < (int)(V * sizeof(T)) / 16; ++q) {
@@ -119,25 +126,25 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
   };
 
 #if KPERF_PIPELINE
-  // software pipeline: row vy+1 is fetched before row vy is computed
-  Rows cur = fetch(vy0);
-  for (int vb = vy0; vb < vy1; vb += NWIN) {
+  // software pipeline: row i+1 is fetched before row i is computed
+  Rows cur = fetch(0);
+  for (int ib = 0; ib < nv; ib += NWIN) {
     auto unrolled = [&](auto uc) {
-      const int vy = vb + decltype(uc)::value;
-      if (vy < vy1) {
+      const int i = ib + decltype(uc)::value;
+      if (i < nv) {
         Rows nxt;
-        if (vy + 1 < vy1) nxt = fetch(vy + 1);
-        compute(uc, cur, vy);
+        if (i + 1 < nv) nxt = fetch(i + 1);
+        compute(uc, cur, vy0 + i);
         cur = nxt;
       }
     };
     static_for<0, NWIN>(unrolled);
   }
 #else
-  for (int vb = vy0; vb < vy1; vb += NWIN) {
+  for (int ib = 0; ib < nv; ib += NWIN) {
     auto unrolled = [&](auto uc) {
-      const int vy = vb + decltype(uc)::value;
-      if (vy < vy1) compute(uc, fetch(vy), vy);
+      const int i = ib + decltype(uc)::value;
+      if (i < nv) compute(uc, fetch(i), vy0 + i);  // (vy only matters to the fused Gauss-Sobel)
     };
     static_for<0, NWIN>(unrolled);
   }
@@ -184,7 +191,7 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : App:
   T* ring = reinterpret_cast<T*>(smem + bar_bytes);
   const int slot_elems = p.row_elems * App::NIN;
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
-  const int nrec = p.seg_h + 2 * kMaxVR;
+  const int nrec = p.seg_h + (p.seg_h / max(p.tile1_h, 1) + 1) * 2 * kMaxVR;  // >= n_recipes
   Recipe* rtab = reinterpret_cast<Recipe*>(smem + bar_bytes + (size_t)p.nr * slot_elems * sizeof(T)) +
                  (warp > 0 ? (warp - 1) * nrec : 0);  // one recipe table per consumer warp
   const Mask m{p.num, p.den, p.keep_one};
@@ -223,9 +230,13 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : App:
     if (warp == 0) {  // (Ia) data perforation: only kept samples leave HBM
       producer<T, SCHEME, App::NIN, TW>(p, m, rp, x0, frame, g0, full, empty, ring);
     } else {
-      const int nv = ye - ys + 2 * App::VR;
+      const int nv = n_recipes<SCHEME>(p, ys, ye, App::VR);
       __syncwarp();
-      for (int i = lane; i < nv; i += 32) rtab[i] = make_recipe<SCHEME, RECON>(p, m, rp, ys - App::VR + i);
+      for (int i = lane; i < nv; i += 32) {
+        int emit;
+        const int y = virtual_row<SCHEME>(p, rp, ys, ye, App::VR, i, emit);
+        rtab[i] = make_recipe<SCHEME, RECON>(p, m, rp, y, emit);
+      }
       __syncwarp();
       const int xw = x0 + (warp - 1) * 32 * V;
       if (p.fast_ok && xw + 32 * V <= p.W)
@@ -270,8 +281,9 @@ cudaError_t launch_one(const KParams& p, unsigned grid, size_t smem, cudaStream_
     const long long per_seg = (long long)p.n_strips * p.frames;
     double best = -1.0;
     int best_n = (rows + p.seg_h - 1) / p.seg_h;
+    const int th = SCHEME == S_STENCIL1 ? p.tile1_h : 1;  // Stencil1 segments hold whole tiles
     for (int n = (rows + p.seg_h - 1) / p.seg_h; n <= (rows + 31) / 32 && n <= 4 * best_n + 64; ++n) {
-      const int sh = (rows + n - 1) / n;
+      const int sh = ((rows + n - 1) / n + th - 1) / th * th;
       const int nn = (rows + sh - 1) / sh;
       const long long items = per_seg * nn;
       const long long waves = (items + slots - 1) / slots;
@@ -280,7 +292,7 @@ cudaError_t launch_one(const KParams& p, unsigned grid, size_t smem, cudaStream_
       const double score = fill * halo;
       if (score > best + 1e-9) { best = score; best_n = nn; }
     }
-    q.seg_h = (rows + best_n - 1) / best_n;
+    q.seg_h = ((rows + best_n - 1) / best_n + th - 1) / th * th;
     q.n_segs = (rows + q.seg_h - 1) / q.seg_h;
     grid = (unsigned)((long long)q.n_strips * q.n_segs * q.frames);
   }
@@ -299,6 +311,10 @@ cudaError_t launch_app(int scheme, int recon, const KParams& p, unsigned grid, s
     case S_COL * 2 + R_LI: return launch_one<App, S_COL, R_LI, NCW>(p, grid, smem, s);
     case S_CHECKER * 2 + R_NN: return launch_one<App, S_CHECKER, R_NN, NCW>(p, grid, smem, s);
     case S_CHECKER * 2 + R_LI: return launch_one<App, S_CHECKER, R_LI, NCW>(p, grid, smem, s);
+    case S_STENCIL1 * 2 + R_NN:
+    case S_STENCIL1 * 2 + R_LI:
+      if constexpr (App::NIN == 1 && App::VR <= 2) return launch_one<App, S_STENCIL1, R_NN, NCW>(p, grid, smem, s);
+      break;
   }
   return cudaErrorInvalidValue;
 }

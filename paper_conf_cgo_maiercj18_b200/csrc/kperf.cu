@@ -48,7 +48,7 @@ struct perf_plan_s {
   int app, W, H, radius, scheme, recon;
   perf_rate rate;
   long long batch = 1, iters = 1, granule_bytes = 128, global_h = -1, band_y0 = 0, tile_w = kp::kNCW, tile_h = 0,
-            metric = 0, loader = 0, ring = 0;
+            metric = 0, loader = 0, ring = 0, tile1_w = 16, tile1_h = 16;
   double* d_err = nullptr;
   float* d_tmp = nullptr;
   size_t tmp_elems = 0;
@@ -85,7 +85,8 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   const int TW = NCW * 32 * V;
   const int Hg = P->global_h > 0 ? (int)P->global_h : P->H;
   int scheme = P->scheme;
-  if (P->rate.num == 0) scheme = PERF_SCHEME_NONE;
+  if (P->rate.num == 0 && scheme != PERF_SCHEME_STENCIL1) scheme = PERF_SCHEME_NONE;
+  const bool s1 = scheme == PERF_SCHEME_STENCIL1;
   std::memset(&k, 0, sizeof k);
   k.in = in;
   k.in2 = in2;
@@ -100,23 +101,26 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   k.out_row0 = out_row0;
   k.y_begin = y_begin;
   k.y_end = y_end;
-  k.num = scheme == PERF_SCHEME_NONE ? 0 : P->rate.num;
-  k.den = scheme == PERF_SCHEME_NONE ? 1 : P->rate.den;
+  k.num = (scheme == PERF_SCHEME_NONE || s1) ? 0 : P->rate.num;
+  k.den = (scheme == PERF_SCHEME_NONE || s1) ? 1 : P->rate.den;
+  k.tile1_w = (int)P->tile1_w;
+  k.tile1_h = (int)P->tile1_h;
   k.keep_one = (k.num == k.den - 1) ? 1 : 0;
   const int G = (int)(P->granule_bytes / es);
   k.G = G < 1 ? 1 : G;
-  k.fast_ok = (scheme == PERF_SCHEME_NONE || scheme == PERF_SCHEME_ROW || (k.G % V) == 0) ? 1 : 0;
-  const bool chunk_uniform = scheme == PERF_SCHEME_NONE || scheme == PERF_SCHEME_ROW || (k.G % CV) == 0;
+  const bool rowwise = scheme == PERF_SCHEME_NONE || scheme == PERF_SCHEME_ROW || s1;  // whole rows kept
+  k.fast_ok = (rowwise || (k.G % V) == 0) ? 1 : 0;
+  const bool chunk_uniform = rowwise || (k.G % CV) == 0;
   const bool aligned = ((reinterpret_cast<uintptr_t>(in) | reinterpret_cast<uintptr_t>(out) |
                          reinterpret_cast<uintptr_t>(in2)) & 15) == 0;
   k.vec_io = (P->W % CV == 0) && aligned ? 1 : 0;
   int loader = (int)P->loader;
   if (loader == kp::L_AUTO) {
     if (!k.vec_io) loader = kp::L_SCALAR;
-    else if (scheme == PERF_SCHEME_NONE || scheme == PERF_SCHEME_ROW) loader = kp::L_BULK;
+    else if (rowwise) loader = kp::L_BULK;
     else loader = chunk_uniform ? kp::L_ASYNC16 : kp::L_SCALAR;
   }
-  if (loader == kp::L_BULK && !(k.vec_io && (scheme == PERF_SCHEME_NONE || scheme == PERF_SCHEME_ROW)))
+  if (loader == kp::L_BULK && !(k.vec_io && rowwise))
     return fail(PERF_ERR_UNSUPPORTED, "loader BULK needs the row/none scheme, W % V == 0 and 16-B aligned buffers");
   if (loader == kp::L_ASYNC16 && !(k.vec_io && chunk_uniform))
     return fail(PERF_ERR_UNSUPPORTED, "loader ASYNC16 needs W*sizeof(T) % 16 == 0, aligned buffers, G*sizeof(T) % 16 == 0");
@@ -136,14 +140,16 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   const int nin = P->app == PERF_APP_HOTSPOT ? 2 : 1;
   const size_t slot_bytes = (size_t)k.row_elems * nin * es;
   auto bar_bytes = [](int n) { return (size_t)((2 * n * 8 + 127) & ~127); };
-  const size_t rec_bytes0 = (size_t)NCW * ((P->tile_h > 0 ? P->tile_h : 128) + 2 * kp::kMaxVR) * sizeof(kp::Recipe);
+  int seg = (int)(P->tile_h > 0 ? P->tile_h : 128);
+  if (s1) seg = (seg + k.tile1_h - 1) / k.tile1_h * k.tile1_h;  // whole Stencil1 tiles per segment
+  const size_t rec_bytes0 =
+      (size_t)NCW * (seg + (seg / k.tile1_h + 1) * 2 * kp::kMaxVR) * sizeof(kp::Recipe);
   while (nr > next_pow2(hold + 1) && bar_bytes(nr) + nr * slot_bytes + rec_bytes0 > 200 * 1024) nr >>= 1;
   k.nr = nr;
   k.nr_log2 = log2i(nr);
-  k.seg_h = (int)(P->tile_h > 0 ? P->tile_h : 128);
+  k.seg_h = seg;
   k.seg_auto = P->tile_h > 0 ? 0 : 1;
-  const size_t recipe_bytes = (size_t)NCW * (k.seg_h + 2 * kp::kMaxVR) * sizeof(kp::Recipe);
-  smem = bar_bytes(nr) + (size_t)nr * slot_bytes + recipe_bytes;
+  smem = bar_bytes(nr) + (size_t)nr * slot_bytes + rec_bytes0;
   if (smem > 227 * 1024) return fail(PERF_ERR_UNSUPPORTED, "shared-memory ring + recipes exceed 227 KB");
   k.n_strips = (P->W + TW - 1) / TW;
   k.n_segs = (y_end - y_begin + k.seg_h - 1) / k.seg_h;
@@ -169,7 +175,7 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
 }
 
 static cudaError_t dispatch(const perf_plan_s* P, const KParams& k, unsigned grid, size_t smem, cudaStream_t s) {
-  int scheme = P->rate.num == 0 ? PERF_SCHEME_NONE : P->scheme;
+  int scheme = (P->rate.num == 0 && P->scheme != PERF_SCHEME_STENCIL1) ? PERF_SCHEME_NONE : P->scheme;
   const int rc = P->recon;
   switch (P->app) {
     case PERF_APP_GAUSSIAN:
@@ -203,7 +209,7 @@ perf_status perf_plan(perf_plan_t* plan, perf_app app, int W, int H, int radius,
   if (!plan) return fail(PERF_ERR_INVALID_ARG, "plan is NULL");
   *plan = nullptr;
   if (app < PERF_APP_GAUSSIAN || app > PERF_APP_INVERSION) return fail(PERF_ERR_INVALID_ARG, "bad app");
-  if (scheme < PERF_SCHEME_NONE || scheme > PERF_SCHEME_CHECKER) return fail(PERF_ERR_INVALID_ARG, "bad scheme");
+  if (scheme < PERF_SCHEME_NONE || scheme > PERF_SCHEME_STENCIL1) return fail(PERF_ERR_INVALID_ARG, "bad scheme");
   if (recon != PERF_RECON_NN && recon != PERF_RECON_LINEAR) return fail(PERF_ERR_INVALID_ARG, "bad recon");
   if (W < 1 || H < 1) return fail(PERF_ERR_INVALID_ARG, "W and H must be >= 1");
   bool r_ok = false;
@@ -219,8 +225,10 @@ perf_status perf_plan(perf_plan_t* plan, perf_app app, int W, int H, int radius,
   if (rate.den < 1 || rate.den > 8) return fail(PERF_ERR_INVALID_ARG, "rate.den must be in [1, 8]");
   if (!(rate.num == 0 || rate.num == 1 || rate.num == rate.den - 1) || rate.num >= rate.den)
     return fail(PERF_ERR_INVALID_ARG, "rate.num must be 0, 1 or den-1 (and < den)");
-  if (scheme == PERF_SCHEME_NONE && rate.num != 0)
-    return fail(PERF_ERR_INVALID_ARG, "scheme NONE needs rate.num == 0");
+  if ((scheme == PERF_SCHEME_NONE || scheme == PERF_SCHEME_STENCIL1) && rate.num != 0)
+    return fail(PERF_ERR_INVALID_ARG, "schemes NONE and STENCIL1 need rate.num == 0");
+  if (scheme == PERF_SCHEME_STENCIL1 && (app == PERF_APP_HOTSPOT || app == PERF_APP_GAUSS_SOBEL))
+    return fail(PERF_ERR_UNSUPPORTED, "STENCIL1 is provided for Gaussian, Sobel, Median and Inversion");
   if (scheme == PERF_SCHEME_CHECKER && rate.num > 0 && H < rate.den)
     return fail(PERF_ERR_INVALID_ARG, "checker scheme needs H >= den");
   perf_plan_s* p = new (std::nothrow) perf_plan_s();
@@ -283,6 +291,17 @@ perf_status perf_plan_set(perf_plan_t p, int key, long long v) {
       return PERF_OK;
     case PERF_KEY_HALO_ROWS:
       return fail(PERF_ERR_INVALID_ARG, "HALO_ROWS is read-only");
+    case PERF_KEY_TILE1_W: {
+      const long long vmax = p->app == PERF_APP_MEDIAN ? 512 : 256;
+      if (v < 16 || v > vmax || (v & (v - 1)))
+        return fail(PERF_ERR_INVALID_ARG, "TILE1_W must be a power of two in [16, 256] (u8: 512)");
+      p->tile1_w = v;
+      return PERF_OK;
+    }
+    case PERF_KEY_TILE1_H:
+      if (v < 1 || v > 1024) return fail(PERF_ERR_INVALID_ARG, "TILE1_H must be in [1, 1024]");
+      p->tile1_h = v;
+      return PERF_OK;
   }
   return fail(PERF_ERR_INVALID_ARG, "unknown key");
 }
@@ -301,6 +320,8 @@ perf_status perf_plan_get(perf_plan_t p, int key, long long* v) {
     case PERF_KEY_LOADER: *v = p->loader; return PERF_OK;
     case PERF_KEY_RING: *v = p->ring; return PERF_OK;
     case PERF_KEY_HALO_ROWS: *v = band_halo(p); return PERF_OK;
+    case PERF_KEY_TILE1_W: *v = p->tile1_w; return PERF_OK;
+    case PERF_KEY_TILE1_H: *v = p->tile1_h; return PERF_OK;
   }
   return fail(PERF_ERR_INVALID_ARG, "unknown key");
 }

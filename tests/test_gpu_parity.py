@@ -347,3 +347,34 @@ def test_c5_frames_sampled():
         xs, ys = _samples(W, H, 300, 10 + b)
         want = oracle.run_pixels(prm, img, xs, ys)
         assert_close("gauss_sobel", 2, out[b].cpu().numpy()[ys, xs], want)
+
+
+# ---------------------------------------------------------------------------
+# NEXT-1: Stencil1 -- tile interior loaded, halo NN from the tile
+@pytest.mark.parametrize("app,r", [("gaussian", 1), ("gaussian", 2), ("sobel", 1), ("sobel", 2), ("inversion", 0),
+                                   ("median", 1)])
+@pytest.mark.parametrize("tile", [(16, 16), (32, 8), (64, 4), (256, 1), (16, 5), (128, 33)])
+def test_stencil1_parity(app, r, tile):
+    u8 = app == "median"
+    W, H = (4200, 140) if u8 else (1100, 300)
+    img = synth.image("natural", 41, W, H, np.uint8 if u8 else np.float32)
+    got = gpu_run(app, r, img, "stencil1", (0, 1), "nn", tile1_w=tile[0], tile1_h=tile[1])
+    want = oracle.run(oracle.params(app, W, H, r, "stencil1", (0, 1), "nn", tile=tile), img)
+    assert_close(app, r, got, want)
+
+
+@pytest.mark.parametrize("shape", [(1, 1), (7, 3), (130, 2), (513, 129), (1027, 33)])
+def test_stencil1_ragged(shape):
+    W, H = shape
+    img = synth.image("pattern", 43, W, H)
+    for tile in [(16, 16), (32, 7)]:
+        got = gpu_run("gaussian", 2, img, "stencil1", (0, 1), "nn", tile1_w=tile[0], tile1_h=tile[1])
+        want = oracle.run(oracle.params("gaussian", W, H, 2, "stencil1", (0, 1), "nn", tile=tile), img)
+        assert_close("gaussian", 2, got, want)
+
+
+def test_stencil1_whole_image_tile_is_exact():
+    W, H = 250, 100
+    img = synth.image("natural", 44, W, H)
+    ex = gpu_run("sobel", 1, img, "none", (0, 1), "nn")
+    assert np.array_equal(gpu_run("sobel", 1, img, "stencil1", (0, 1), "nn", tile1_w=256, tile1_h=128), ex)
