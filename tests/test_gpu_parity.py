@@ -378,3 +378,25 @@ def test_stencil1_whole_image_tile_is_exact():
     img = synth.image("natural", 44, W, H)
     ex = gpu_run("sobel", 1, img, "none", (0, 1), "nn")
     assert np.array_equal(gpu_run("sobel", 1, img, "stencil1", (0, 1), "nn", tile1_w=256, tile1_h=128), ex)
+
+
+# ---------------------------------------------------------------------------
+# NEXT-2: the paper's error orderings reproduced through the GPU path
+def test_paper_orderings_on_gpu():
+    """Sec. 6.3 and Fig. 7 (:790-800) on synthetic stand-ins"""
+    W = H = 512
+    def mre(app, r, img, scheme, rate, recon, **k):
+        ex = gpu_run(app, r, img, "none", (0, 1), "nn")
+        ap = gpu_run(app, r, img, scheme, rate, recon, **k)
+        with kp.Plan(app, W, H, r) as p:
+            return p.error(torch.from_numpy(ex).cuda(), torch.from_numpy(ap).cuda())[0]
+    nat = synth.image("natural", 0x5EED3100, W, H)
+    for app, r in (("gaussian", 1), ("inversion", 0)):
+        r1n, r2n = mre(app, r, nat, "row", (1, 2), "nn"), mre(app, r, nat, "row", (3, 4), "nn")
+        r1l = mre(app, r, nat, "row", (1, 2), "li")
+        assert r2n > r1n > r1l and r1n < 0.04  # :822-833
+    s1 = mre("gaussian", 1, nat, "stencil1", (0, 1), "nn")
+    assert s1 < 0.01 and s1 < mre("gaussian", 1, nat, "row", (1, 2), "nn")  # :824-826, :833-834
+    errs = [mre("median", 1, synth.image(c, 0x5EED3200, W, H, np.uint8), "row", (1, 2), "nn")
+            for c in ("flat", "natural", "pattern")]
+    assert errs[0] < errs[1] < errs[2]  # Fig. 7: 0.12% < 5.05% < 19.32%
