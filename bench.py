@@ -90,12 +90,13 @@ _bwp = None
 _mix_cache = {}
 
 
-def mixed_peak_gbs(in_ptr, out_ptr, out_bytes, scheme, rate, gran_bytes=128, n_in=1, stream=0):
-    """GB/s a plain streaming kernel reaches with the same read/write mix as a
-    perforated stencil (tools/bwprobe.cu, measured on this box): every output
-    byte written once, the kept fraction of the input read, in 16-KB rows (row
-    scheme / exact) or gran_bytes cells (column / checker).  Algorithmic bytes
-    over the probe's time, so it is directly comparable to roofline.achieved."""
+def mixed_peak_gbs(in_ptr, out_ptr, out_bytes, scheme, rate, gran_bytes=128, n_in=1, stream=0, pitch_bytes=16384):
+    """GB/s a plain streaming kernel reaches with the same read/write mix and the
+    same per-CTA footprint as a perforated stencil (tools/bwprobe.cu, measured on
+    this box): every output byte written once, the kept fraction of the input read
+    (whole rows for the row scheme / exact, gran_bytes cells for column /
+    checker), each CTA streaming 4-KB x 128-row blocks, best of 4 / 8 CTAs per SM.
+    Algorithmic bytes over the probe's time: comparable to roofline.achieved."""
     global _bwp
     import ctypes
     if _bwp is None:
@@ -103,16 +104,20 @@ def mixed_peak_gbs(in_ptr, out_ptr, out_bytes, scheme, rate, gran_bytes=128, n_i
         _bwp.bwp_time_ms.restype = ctypes.c_float
         _bwp.bwp_time_ms.argtypes = [ctypes.c_void_p, ctypes.c_void_p, ctypes.c_longlong, ctypes.c_int,
                                      ctypes.c_int, ctypes.c_int, ctypes.c_int, ctypes.c_int, ctypes.c_void_p]
+        _bwp.bwp_block_ms.restype = ctypes.c_float
+        _bwp.bwp_block_ms.argtypes = [ctypes.c_void_p, ctypes.c_void_p, ctypes.c_longlong, ctypes.c_longlong,
+                                      ctypes.c_int, ctypes.c_int, ctypes.c_int, ctypes.c_int, ctypes.c_int,
+                                      ctypes.c_int, ctypes.c_int, ctypes.c_void_p]
     num, den = rate
     if scheme == "none" or num == 0:
         kn, kd = 1, 1
     else:
         kd = den
         kn = den - num
-    unit = 16384 if scheme in ("none", "row") else gran_bytes
-    key = (out_bytes, kn, kd, unit, n_in)
+    unit = pitch_bytes if scheme in ("none", "row") else gran_bytes
+    key = (out_bytes, kn, kd, unit, n_in, pitch_bytes)
     if key not in _mix_cache:
-        ms = _bwp.bwp_time_ms(in_ptr, out_ptr, out_bytes, kn, kd, unit, n_in, 5, stream)
+        ms = _bwp.bwp_block_ms(in_ptr, out_ptr, out_bytes, pitch_bytes, 4096, 128, kn, kd, unit, n_in, 3, stream)
         k = kn / kd
         _mix_cache[key] = (n_in * k + 1.0) * out_bytes / (ms * 1e-3) / 1e9 if ms > 0 else None
     return _mix_cache[key]
@@ -372,7 +377,7 @@ def main():
                    "frac": alu_ach / alu_peak, "ops_per_px": ops_px,
                    "peak_derivation": "148 SM x 4 SMSP x 16 lanes/clk (ALU pipe, 1 warp-inst / 2 clk) x 1965 MHz"}
         pmix = mixed_peak_gbs(x.data_ptr(), yex.data_ptr(), px_step * es, cfg["scheme"], cfg["rate"], G,
-                              stream=stream.cuda_stream) if not u8 else None
+                              stream=stream.cuda_stream, pitch_bytes=W * es) if not u8 else None
         result = {
             "metric": METRIC, "value": value, "unit": unit, "n_gpus": ws, "steps": args.steps,
             "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True, "scaling": "weak",
@@ -389,7 +394,7 @@ def main():
                          "frac": achieved / peak, "traffic": tr, "kernel": kkey,
                          "algorithmic_bytes_per_launch": algo_b, "peak_source": peak_src,
                          "peak_mix": pmix, "frac_mix": achieved / pmix if pmix else None,
-                         "peak_mix_source": "tools/bwprobe.cu on this box: plain stream, same read/write mix"},
+                         "peak_mix_source": "tools/bwprobe.cu on this box: plain stream, same read/write mix and CTA footprint"},
             "clocks": clk.summary(),
             "gpu_launches": args.steps,
         }
@@ -530,7 +535,7 @@ def bench_hotspot(args, cfg, ws, rank, local, stream, peak, peak_src):
     achieved = algo_b / (ms * 1e-3) / 1e9
     scratch = torch.empty((2, h, W), device="cuda")
     pmix = mixed_peak_gbs(scratch.data_ptr(), out_ex.data_ptr(), W * h * 4, cfg["scheme"], cfg["rate"], 128,
-                          n_in=2, stream=stream.cuda_stream)
+                          n_in=2, stream=stream.cuda_stream, pitch_bytes=W * 4)
     del scratch
     return {"metric": METRIC, "value": cells / (ms * 1e-3) / 1e6, "unit": "Mcell-updates/s", "n_gpus": ws,
             "steps": args.steps, "warmup": 1, "ms_per_step": ms, "higher_is_better": True,

@@ -3,6 +3,8 @@
 #pragma once
 #include <cuda_runtime.h>
 
+#include <cstdio>
+
 #include "apps.cuh"
 #include "engine.cuh"
 
@@ -73,38 +75,51 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
     int emit;
   };
   // fetch: recipe, ring release/wait, rebuild from shared memory (a1/a2)
+  // fetch: recipe, ring release/wait, rebuild from shared memory (a1/a2).
+  // After the first row, a row needs at most one more ring row and frees at
+  // most one (every scheme's recipes advance by <= 1), so the waits are ifs.
   auto fetch = [&](int i) {
     Rows r;
     const Recipe rec = rtab[i];
     const int need_hi = g0 + (rec.need & 0x7FFF), need_lo = g0 + (int)((uint32_t)rec.need >> 16);
     r.emit = (rec.need >> 15) & 1;
-    // release ring slots no later row reads (earlier rows are already in registers)
-#pragma unroll 1
-    while (released < need_lo) {
-      __syncwarp();
-      if (lane == 0) mbar_arrive_u32(empty_u32 + 8 * (released & nmask));
+    if (released < need_lo) {  // every lane arrives (empty barrier count = 32 x active warps)
+      mbar_arrive_u32(empty_u32 + 8 * (released & nmask));
       ++released;
     }
-#pragma unroll 1
-    while (ready < need_hi) {
+    if (ready < need_hi) {
       ++ready;
       mbar_wait_u32(full_u32 + 8 * (ready & nmask), (ready >> p.nr_log2) & 1);
     }
     if (FAST) {
       r.c = rebuild_frag<T, V, SCHEME, RECON>(p, m, rp, rec, cc, ring, slot_elems, ccol, xc, base);
       if (App::NIN > 1) r.c2 = rebuild_frag<T, V, SCHEME, RECON>(p, m, rp, rec, cc, ring2, slot_elems, ccol, xc, base);
-      if (emode == 0) r.e = rebuild_frag<T, EW, SCHEME, RECON>(p, m, rp, rec, ce, ring, slot_elems, ecol, ex, base);
-      else if (emode == 1) r.e = Frag<T, EW>::splat(r.c.get(0));
-      else if (emode == 2) r.e = Frag<T, EW>::splat(r.c.get(V - 1));
-      else r.e = rebuild_frag_generic<T, EW, SCHEME, RECON>(p, m, rp, ctx_of<SCHEME>(rec), ring, slot_elems, ex, base);
+      // edge fragment: loaded (inside the image) or the clamped border sample -- selects, no branch
+      const Frag<T, EW> el = rebuild_frag<T, EW, SCHEME, RECON>(p, m, rp, rec, ce, ring, slot_elems, ecol, ex, base);
+      const Frag<T, EW> eb = Frag<T, EW>::splat(emode == 1 ? r.c.get(0) : r.c.get(V - 1));
+      r.e = emode == 0 ? el : eb;
     } else {
       const RowCtx rc = ctx_of<SCHEME>(rec);
       r.c = rebuild_frag_generic<T, V, SCHEME, RECON>(p, m, rp, rc, ring, slot_elems, xc, base);
       r.e = rebuild_frag_generic<T, EW, SCHEME, RECON>(p, m, rp, rc, ring, slot_elems, ex, base);
       if (App::NIN > 1) r.c2 = rebuild_frag_generic<T, V, SCHEME, RECON>(p, m, rp, rc, ring2, slot_elems, xc, base);
+#ifdef KPERF_DEBUG_EDGE
+      if (lane == 31 && i < 6 && sizeof(T) == 4)
+        printf("dbg blk %d warp %d i %d y %d ex %d base %d slot %d e %f %f c7 %f ring516 %f\n", blockIdx.x,
+               threadIdx.x >> 5, i, rec.y, ex, base, rc.slot_c, (double)r.e.get(0), (double)r.e.get(EW - 1),
+               (double)r.c.get(V - 1), (double)ring[rc.slot_c * slot_elems + 516]);
+#endif
     }
     return r;
   };
+  {  // the first row may need several ring rows
+    const int need0 = g0 + (rtab[0].need & 0x7FFF);
+#pragma unroll 1
+    while (ready < need0 - 1) {
+      ++ready;
+      mbar_wait_u32(full_u32 + 8 * (ready & nmask), (ready >> p.nr_log2) & 1);
+    }
+  }
   // compute: the unchanged stencil on the rebuilt row (a3) and the store
   auto compute = [&](auto uc, const Rows& r, int vy) {
     constexpr int U = decltype(uc)::value;
@@ -156,10 +171,8 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
     ++ready;
     mbar_wait_u32(full_u32 + 8 * (ready & nmask), (ready >> p.nr_log2) & 1);
   }
-  __syncwarp();
 #pragma unroll 1
-  for (; released < g_end; ++released)
-    if (lane == 0) mbar_arrive_u32(empty_u32 + 8 * (released & nmask));
+  for (; released < g_end; ++released) mbar_arrive_u32(empty_u32 + 8 * (released & nmask));
 }
 
 template <class App, int SCHEME, int RECON, int NCW>
@@ -206,7 +219,7 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : App:
   if (threadIdx.x == 0) {
     for (int s = 0; s < p.nr; ++s) {
       mbar_init(&full[s], p.loader == L_BULK ? 1u : 32u);
-      mbar_init(&empty[s], (uint32_t)nact);
+      mbar_init(&empty[s], (uint32_t)(32 * nact));  // every consumer lane arrives
     }
     mbar_fence_init();
   }
@@ -239,7 +252,11 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : App:
       }
       __syncwarp();
       const int xw = x0 + (warp - 1) * 32 * V;
-      if (p.fast_ok && xw + 32 * V <= p.W)
+      // fast path: every lane chunk inside the image, and the right edge fragment
+      // either inside or starting exactly at W (then it is the clamped border)
+      const int exr = xw + 32 * V;
+      const bool edges_ok = (exr + App::EW <= p.W) || (exr == p.W);
+      if (p.fast_ok && xw + 32 * V <= p.W && edges_ok)
         consumer_fast<App, SCHEME, RECON, NCW>(p, m, rp, x0, frame, ys, ye, g0, full_u32, empty_u32, ring,
                                                slot_elems, rtab);
       else

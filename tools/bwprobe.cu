@@ -9,6 +9,28 @@
 
 #include <cstdint>
 
+// block pattern: each CTA streams blocks of bw4 x bh (16-B units x rows) of a
+// pitch4-wide image, the footprint of one perforated-stencil CTA (strip x segment)
+__global__ void bwp_block(const float4* __restrict__ in, float4* __restrict__ out, int rows, int pitch4, int bw4,
+                          int bh, int keep_num, int keep_den, int unit4, int n_in, long long plane4) {
+  const int nbx = (pitch4 + bw4 - 1) / bw4, nby = (rows + bh - 1) / bh, nb = nbx * nby;
+  for (int b = blockIdx.x; b < nb; b += gridDim.x) {
+    const int bx = b % nbx, by = b / nbx;
+    const int c1 = min(bw4, pitch4 - bx * bw4);
+    for (int r = by * bh; r < min(rows, by * bh + bh); ++r)
+      for (int c = threadIdx.x; c < c1; c += blockDim.x) {
+        const long long i = (long long)r * pitch4 + bx * bw4 + c;
+        const long long u = unit4 >= pitch4 ? r : i / unit4;  // row-like units, or granules along the row
+        float4 v = make_float4(1.f, 2.f, 3.f, 4.f);
+        if ((int)(u % keep_den) < keep_num) {
+          v = __ldcs(in + i);
+          if (n_in > 1) v.x += __ldcs(in + plane4 + i).x;
+        }
+        __stcs(out + i, v);
+      }
+  }
+}
+
 __global__ void bwp_mix(const float4* __restrict__ in, float4* __restrict__ out, long long n4, int keep_num,
                         int keep_den, int unit4, int n_in) {
   for (long long i = blockIdx.x * (long long)blockDim.x + threadIdx.x; i < n4;
@@ -27,6 +49,37 @@ __global__ void bwp_mix(const float4* __restrict__ in, float4* __restrict__ out,
 }
 
 extern "C" {
+// Block-pattern ceiling: pitch_bytes-wide rows (the image width), blocks of
+// block_bytes x block_rows per CTA, best of 4 / 8 CTAs per SM.  Returns ms.
+float bwp_block_ms(const void* in, void* out, long long n_out_bytes, long long pitch_bytes, int block_bytes,
+                   int block_rows, int keep_num, int keep_den, int unit_bytes, int n_in, int reps, void* stream) {
+  cudaStream_t s = (cudaStream_t)stream;
+  const int pitch4 = (int)(pitch_bytes / 16), rows = (int)(n_out_bytes / pitch_bytes);
+  const int bw4 = block_bytes / 16, unit4 = unit_bytes >= pitch_bytes ? pitch4 : (unit_bytes / 16 > 0 ? unit_bytes / 16 : 1);
+  int dev = 0, sms = 148;
+  cudaGetDevice(&dev);
+  cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
+  cudaEvent_t e0, e1;
+  cudaEventCreate(&e0);
+  cudaEventCreate(&e1);
+  float best = 1e30f;
+  for (int cps : {4, 8}) {
+    for (int r = 0; r < reps + 1; ++r) {
+      cudaEventRecord(e0, s);
+      bwp_block<<<sms * cps, 256, 0, s>>>((const float4*)in, (float4*)out, rows, pitch4, bw4, block_rows, keep_num,
+                                          keep_den, unit4, n_in, n_out_bytes / 16);
+      cudaEventRecord(e1, s);
+      cudaEventSynchronize(e1);
+      float ms;
+      cudaEventElapsedTime(&ms, e0, e1);
+      if (r >= 1 && ms < best) best = ms;
+    }
+  }
+  cudaEventDestroy(e0);
+  cudaEventDestroy(e1);
+  return cudaGetLastError() == cudaSuccess ? best : -1.f;
+}
+
 // Time one pass: n_out bytes written, keep_num/keep_den of the input units
 // (unit_bytes each; 16 KB = row-like, 128 B = granule-like) read from n_in
 // arrays of the same size.  Buffers are caller-provided device memory:
