@@ -49,6 +49,7 @@ struct KParams {
   int fast_ok;               // every V-chunk lies in one mask cell (G % V == 0 or row scheme)
   int vec_io;                // W % V == 0 and 16-B aligned buffers
   int tile1_w, tile1_h;      // Stencil1 work-group tile
+  int nrec;                  // recipe-table entries per consumer warp (>= n_recipes of a segment)
   float sdc, rx1, ry1, rz1, amb;  // Hotspot (Rodinia) coefficients
 };
 

@@ -204,7 +204,7 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : App:
   T* ring = reinterpret_cast<T*>(smem + bar_bytes);
   const int slot_elems = p.row_elems * App::NIN;
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
-  const int nrec = p.seg_h + (p.seg_h / max(p.tile1_h, 1) + 1) * 2 * kMaxVR;  // >= n_recipes
+  const int nrec = p.nrec;
   Recipe* rtab = reinterpret_cast<Recipe*>(smem + bar_bytes + (size_t)p.nr * slot_elems * sizeof(T)) +
                  (warp > 0 ? (warp - 1) * nrec : 0);  // one recipe table per consumer warp
   const Mask m{p.num, p.den, p.keep_one};

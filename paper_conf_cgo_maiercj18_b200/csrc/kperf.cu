@@ -142,8 +142,9 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   auto bar_bytes = [](int n) { return (size_t)((2 * n * 8 + 127) & ~127); };
   int seg = (int)(P->tile_h > 0 ? P->tile_h : 128);
   if (s1) seg = (seg + k.tile1_h - 1) / k.tile1_h * k.tile1_h;  // whole Stencil1 tiles per segment
-  const size_t rec_bytes0 =
-      (size_t)NCW * (seg + (seg / k.tile1_h + 1) * 2 * kp::kMaxVR) * sizeof(kp::Recipe);
+  // recipes per segment: seg + 2 VR rows, Stencil1: every tile restarts its window
+  k.nrec = s1 ? seg + (seg / k.tile1_h + 1) * 2 * kp::kMaxVR : seg + 2 * kp::kMaxVR;
+  const size_t rec_bytes0 = (size_t)NCW * k.nrec * sizeof(kp::Recipe);
   while (nr > next_pow2(hold + 1) && bar_bytes(nr) + nr * slot_bytes + rec_bytes0 > 200 * 1024) nr >>= 1;
   k.nr = nr;
   k.nr_log2 = log2i(nr);
