@@ -101,7 +101,8 @@ enum {
   PERF_KEY_RING = 10,          /* shared-memory ring depth in rows (0 = auto) */
   PERF_KEY_HALO_ROWS = 11,     /* read-only: rows a Hotspot band exchanges with each neighbour per step */
   PERF_KEY_TILE1_W = 12,       /* STENCIL1 tile width: power of two, 16..256 (fp32) / 16..512 (u8); default 16 */
-  PERF_KEY_TILE1_H = 13        /* STENCIL1 tile height, 1..1024; default 16 */
+  PERF_KEY_TILE1_H = 13,       /* STENCIL1 tile height, 1..1024; default 16 */
+  PERF_KEY_PRODUCER = 14       /* 0 auto = 1 dedicated producer warp; 2 bulk rows issued by consumer warp 0 */
 };
 
 /* Create a plan.  Validates: W, H >= 1; radius allowed for the app (Gaussian,

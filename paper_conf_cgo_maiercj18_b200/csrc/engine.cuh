@@ -50,6 +50,7 @@ struct KParams {
   int vec_io;                // W % V == 0 and 16-B aligned buffers
   int tile1_w, tile1_h;      // Stencil1 work-group tile
   int nrec;                  // recipe-table entries per consumer warp (>= n_recipes of a segment)
+  int inline_prod;           // bulk loader issued by consumer warp 0 (no dedicated producer warp)
   float sdc, rx1, ry1, rz1, amb;  // Hotspot (Rodinia) coefficients
 };
 
@@ -210,6 +211,21 @@ __device__ __forceinline__ int row_of_idx(const Mask& m, const RowPlan& rp, int 
 
 // ---------------------------------------------------------------------------
 // producer warp: fetch the kept part of every needed row into the ring
+// one kept row (and its power row) by TMA-engine bulk copies; lane 0 only
+template <typename T, int SCHEME, int NIN, int TW>
+__device__ __forceinline__ void issue_bulk_row(const KParams& p, const Mask& m, const RowPlan& rp, int x0, int frame,
+                                               int g, int i, uint64_t* full, T* ring) {
+  const int cx0 = max(x0 - p.hx, 0), cx1 = min(x0 + TW + p.hx, p.W);
+  const int slot = g & (p.nr - 1);
+  const int y = row_of_idx<SCHEME>(m, rp, i);
+  const long long roff = (long long)(y - p.in_row0) * p.W + (long long)frame * p.in_fstride;
+  T* dst = ring + slot * p.row_elems * NIN + (cx0 - (x0 - p.hx));
+  const uint32_t b0 = (uint32_t)((cx1 - cx0) * sizeof(T));
+  mbar_arrive_expect_tx(&full[slot], b0 * NIN);
+  bulk_g2s(dst, static_cast<const T*>(p.in) + roff + cx0, b0, &full[slot]);
+  if (NIN > 1) bulk_g2s(dst + p.row_elems, static_cast<const T*>(p.in2) + roff + cx0, b0, &full[slot]);
+}
+
 // g0: global (per-CTA, across work items) index of this item's first load;
 // ring slot = g & (nr-1), fill phase = g >> log2(nr).
 template <typename T, int SCHEME, int NIN, int TW>

@@ -46,7 +46,35 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
   using T = typename App::T;
   constexpr int V = App::V, EW = App::EW, VR = App::VR, NWIN = App::NWIN;
   constexpr int CV = 16 / sizeof(T);  // elements of one 16-B mask-uniform chunk
-  const int lane = threadIdx.x & 31, w = (threadIdx.x >> 5) - 1;
+  constexpr int TW = NCW * 32 * V;
+  const int lane = threadIdx.x & 31, w = (threadIdx.x >> 5) - (p.inline_prod ? 0 : 1);
+  // inline producer (bulk loader): consumer warp 0 issues the kept rows itself
+  const bool issuer = p.inline_prod && w == 0;
+  uint64_t* full_p = reinterpret_cast<uint64_t*>(__cvta_shared_to_generic(full_u32));
+  T* ring_w = const_cast<T*>(ring);
+  int issued = 0;
+  // issue every row whose slot is free (non-blocking); then make sure row `upto` is issued
+  auto issue_ahead = [&](int upto) {
+#pragma unroll 1
+    while (issued < rp.nload) {
+      const int g = g0 + issued;
+      if (g >= p.nr) {
+        const uint32_t par = ((g >> p.nr_log2) - 1) & 1;
+        const uint32_t ea = empty_u32 + 8 * (g & (p.nr - 1));
+        if (issued > upto) {
+          uint32_t ok;
+          asm volatile("{\n .reg .pred q;\n mbarrier.test_wait.parity.shared::cta.b64 q, [%1], %2;\n selp.u32 %0, 1, 0, q;\n}"
+                       : "=r"(ok) : "r"(ea), "r"(par) : "memory");
+          if (!ok) break;
+        } else {
+          mbar_wait_u32(ea, par);
+        }
+      }
+      if (lane == 0)
+        issue_bulk_row<T, SCHEME, App::NIN, TW>(p, m, rp, x0, frame, g, issued, full_p, ring_w);
+      ++issued;
+    }
+  };
   const int xw = x0 + w * 32 * V;
   const int base = x0 - p.hx;
   const int xc = xw + lane * V;
@@ -87,6 +115,7 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
       mbar_arrive_u32(empty_u32 + 8 * (released & nmask));
       ++released;
     }
+    if (issuer) issue_ahead(need_hi - g0);
     if (ready < need_hi) {
       ++ready;
       mbar_wait_u32(full_u32 + 8 * (ready & nmask), (ready >> p.nr_log2) & 1);
@@ -114,6 +143,7 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
   };
   {  // the first row may need several ring rows
     const int need0 = g0 + (rtab[0].need & 0x7FFF);
+    if (issuer) issue_ahead(need0 - g0);
 #pragma unroll 1
     while (ready < need0 - 1) {
       ++ready;
@@ -206,7 +236,7 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : App:
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   const int nrec = p.nrec;
   Recipe* rtab = reinterpret_cast<Recipe*>(smem + bar_bytes + (size_t)p.nr * slot_elems * sizeof(T)) +
-                 (warp > 0 ? (warp - 1) * nrec : 0);  // one recipe table per consumer warp
+                 max(warp - (p.inline_prod ? 0 : 1), 0) * nrec;  // one recipe table per consumer warp
   const Mask m{p.num, p.den, p.keep_one};
   const int n_items = p.n_strips * p.n_segs * p.frames;
 
@@ -224,7 +254,8 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : App:
     mbar_fence_init();
   }
   __syncthreads();
-  if (warp > nact) return;
+  const int cw0 = p.inline_prod ? 0 : 1;  // first consumer warp
+  if (warp - cw0 >= nact) return;
   const uint32_t full_u32 = smem_u32(full), empty_u32 = smem_u32(empty);
 
   const int g0 = 0;  // global load index of the item's first row (one item per CTA)
@@ -240,7 +271,7 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : App:
     const int ys = p.y_begin + seg * p.seg_h;
     const int ye = min(ys + p.seg_h, p.y_end);
     const RowPlan rp = make_row_plan<SCHEME>(p, m, ys, ye, App::VR);
-    if (warp == 0) {  // (Ia) data perforation: only kept samples leave HBM
+    if (!p.inline_prod && warp == 0) {  // (Ia) data perforation: only kept samples leave HBM
       producer<T, SCHEME, App::NIN, TW>(p, m, rp, x0, frame, g0, full, empty, ring);
     } else {
       const int nv = n_recipes<SCHEME>(p, ys, ye, App::VR);
@@ -251,7 +282,7 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : App:
         rtab[i] = make_recipe<SCHEME, RECON>(p, m, rp, y, emit);
       }
       __syncwarp();
-      const int xw = x0 + (warp - 1) * 32 * V;
+      const int xw = x0 + (warp - cw0) * 32 * V;
       // fast path: every lane chunk inside the image, and the right edge fragment
       // either inside or starting exactly at W (then it is the clamped border)
       const int exr = xw + 32 * V;
@@ -288,7 +319,8 @@ cudaError_t launch_one(const KParams& p, unsigned grid, size_t smem, cudaStream_
       int dev = 0;
       cudaGetDevice(&dev);
       cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
-      if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k, 32 * (NCW + 1), smem) != cudaSuccess ||
+      if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k, 32 * (NCW + (p.inline_prod ? 0 : 1)), smem) !=
+              cudaSuccess ||
           per_sm < 1)
         per_sm = 1;
       per_sm_smem = smem;
@@ -313,7 +345,7 @@ cudaError_t launch_one(const KParams& p, unsigned grid, size_t smem, cudaStream_
     q.n_segs = (rows + q.seg_h - 1) / q.seg_h;
     grid = (unsigned)((long long)q.n_strips * q.n_segs * q.frames);
   }
-  k<<<grid, 32 * (NCW + 1), smem, s>>>(q);
+  k<<<grid, 32 * (NCW + (p.inline_prod ? 0 : 1)), smem, s>>>(q);
   return cudaGetLastError();
 }
 

@@ -48,7 +48,7 @@ struct perf_plan_s {
   int app, W, H, radius, scheme, recon;
   perf_rate rate;
   long long batch = 1, iters = 1, granule_bytes = 128, global_h = -1, band_y0 = 0, tile_w = kp::kNCW, tile_h = 0,
-            metric = 0, loader = 0, ring = 0, tile1_w = 16, tile1_h = 16;
+            metric = 0, loader = 0, ring = 0, tile1_w = 16, tile1_h = 16, producer = 0;
   double* d_err = nullptr;
   float* d_tmp = nullptr;
   size_t tmp_elems = 0;
@@ -125,6 +125,10 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   if (loader == kp::L_ASYNC16 && !(k.vec_io && chunk_uniform))
     return fail(PERF_ERR_UNSUPPORTED, "loader ASYNC16 needs W*sizeof(T) % 16 == 0, aligned buffers, G*sizeof(T) % 16 == 0");
   k.loader = loader;
+  // PERF_KEY_PRODUCER 2: bulk rows issued by consumer warp 0 instead of a dedicated
+  // producer warp (frees registers for a 5th CTA/SM but refills the ring only once
+  // per warp-0 row: measured 5% slower on C2, so the dedicated warp is the default)
+  k.inline_prod = (loader == kp::L_BULK && P->producer == 2) ? 1 : 0;
   // halo / apron columns: the lane edge chunk (V) plus, for the column scheme,
   // the distance to the nearest loaded granule on either side (<= den * G)
   int hx = CV;
@@ -303,6 +307,10 @@ perf_status perf_plan_set(perf_plan_t p, int key, long long v) {
       if (v < 1 || v > 1024) return fail(PERF_ERR_INVALID_ARG, "TILE1_H must be in [1, 1024]");
       p->tile1_h = v;
       return PERF_OK;
+    case PERF_KEY_PRODUCER:
+      if (v < 0 || v > 2) return fail(PERF_ERR_INVALID_ARG, "PRODUCER must be 0 (auto), 1 (dedicated) or 2 (inline)");
+      p->producer = v;
+      return PERF_OK;
   }
   return fail(PERF_ERR_INVALID_ARG, "unknown key");
 }
@@ -323,6 +331,7 @@ perf_status perf_plan_get(perf_plan_t p, int key, long long* v) {
     case PERF_KEY_HALO_ROWS: *v = band_halo(p); return PERF_OK;
     case PERF_KEY_TILE1_W: *v = p->tile1_w; return PERF_OK;
     case PERF_KEY_TILE1_H: *v = p->tile1_h; return PERF_OK;
+    case PERF_KEY_PRODUCER: *v = p->producer; return PERF_OK;
   }
   return fail(PERF_ERR_INVALID_ARG, "unknown key");
 }

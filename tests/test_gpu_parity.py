@@ -162,6 +162,15 @@ def test_loaders_and_tiles_give_identical_bits():
                 assert np.array_equal(got, ref), (scheme, ld, th)
 
 
+def test_inline_producer_gives_identical_bits():
+    W, H = 2048, 260
+    img = synth.image("natural", 19, W, H)
+    for scheme, rate, recon in [("row", (1, 2), "li"), ("none", (0, 1), "nn"), ("row", (3, 4), "nn"),
+                                ("stencil1", (0, 1), "nn")]:
+        ref = gpu_run("gaussian", 2, img, scheme, rate, recon)
+        assert np.array_equal(gpu_run("gaussian", 2, img, scheme, rate, recon, producer=2), ref)
+
+
 def test_constant_image_rebuilds_exactly():
     W, H = 700, 150
     img = np.full((H, W), 93.0, dtype=np.float32)
