@@ -241,14 +241,25 @@ __device__ __forceinline__ void producer(const KParams& p, const Mask& m, const 
   const int slot_elems = p.row_elems * NIN;
   const int base = x0 - p.hx;  // global column of ring element 0
 
-  // per-lane chunk phases for the column / checker schemes (row independent)
-  constexpr int KMAX = 8;
-  int gph[KMAX];
+  // 16-B chunks (lane + 32 k) of the row: per lane, a one-hot of the chunk's mask
+  // phase (column / checker cell phase, row independent; 0 = outside the row).
+  // A row's kept phases form a bit mask, so "chunk kept" is one AND and the
+  // copies are predicated LDGSTS with no branches.
+  constexpr int KMAX = 12;
+  uint32_t onehot[KMAX];
 #pragma unroll
   for (int k = 0; k < KMAX; ++k) {
     const int c = cx0 + (lane + 32 * k) * V;
-    gph[k] = (SCHEME == S_COL || SCHEME == S_CHECKER) && c < cx1 ? (c / p.G) % m.den : 0;
+    const bool cell = SCHEME == S_COL || SCHEME == S_CHECKER;
+    onehot[k] = c < cx1 ? (cell ? 1u << ((c / p.G) % m.den) : 1u) : 0u;
   }
+  // kept-phase mask of the column scheme: bit t <=> phase t is loaded
+  uint32_t kmask = 0;
+  for (int t = 0; t < m.den; ++t) kmask |= (uint32_t)m.phase_kept(t) << t;
+  const uint32_t dmask = (1u << m.den) - 1u;
+  const uint32_t lane_dst0 = smem_u32(ring) + (uint32_t)((cx0 - base + lane * V) * (int)sizeof(T));
+  const T* lane_src0 = in + cx0 + lane * V;
+  const T* lane_src1 = in2 + cx0 + lane * V;
 
   for (int i = 0; i < rp.nload; ++i) {
     const int g = g0 + i;
@@ -267,25 +278,22 @@ __device__ __forceinline__ void producer(const KParams& p, const Mask& m, const 
         if (NIN > 1) bulk_g2s(dst + p.row_elems + (px0 - base), in2 + roff + px0, b1, &full[slot]);
       }
     } else if (p.loader == L_ASYNC16) {
-      const int ym = (SCHEME == S_CHECKER) ? y % m.den : 0;
+      // cell (g) of row y is kept iff phase (g + y) % den is (checker), g is (column)
+      uint32_t rmask = 1u;
+      if (SCHEME == S_COL) rmask = kmask;
+      if (SCHEME == S_CHECKER) {
+        const int ym = y % m.den;
+        rmask = ((kmask >> ym) | (kmask << (m.den - ym))) & dmask;
+      }
+      const uint32_t d0 = lane_dst0 + (uint32_t)(slot * slot_elems * (int)sizeof(T));
+      const T* s0 = lane_src0 + roff;
 #pragma unroll
       for (int k = 0; k < KMAX; ++k) {
-        const int c = cx0 + (lane + 32 * k) * V;
-        if (c < cx1) {
-          bool kept = true;
-          if (SCHEME == S_COL) kept = m.phase_kept(gph[k]);
-          if (SCHEME == S_CHECKER) {
-            int t = gph[k] + ym;
-            if (t >= m.den) t -= m.den;
-            kept = m.phase_kept(t);
-          }
-          if (kept) {
-            cp_async16(dst + (c - base), in + roff + c);
-            if (NIN > 1 && c >= px0 && c < px1) cp_async16(dst + p.row_elems + (c - base), in2 + roff + c);
-          }
-        }
+        const uint32_t pk = rmask & onehot[k];
+        cp_async16_if(d0 + k * 32 * 16, s0 + k * 32 * V, pk);
+        if (NIN > 1) cp_async16_if(d0 + (p.row_elems + k * 32 * V) * (int)sizeof(T), lane_src1 + roff + k * 32 * V, pk);
       }
-      for (int c = cx0 + (lane + 32 * KMAX) * V; c < cx1; c += 32 * V) {  // (wide apron; rare)
+      for (int c = cx0 + (lane + 32 * KMAX) * V; c < cx1; c += 32 * V) {  // (very wide apron; rare)
         if (px_kept<SCHEME>(p, m, c, y)) {
           cp_async16(dst + (c - base), in + roff + c);
           if (NIN > 1 && c >= px0 && c < px1) cp_async16(dst + p.row_elems + (c - base), in2 + roff + c);
