@@ -177,96 +177,88 @@ struct AppHotspot {
 };
 
 // ---------------------------------------------------------------------------
-// Gaussian5 -> Sobel3 fused (the C5 pipeline).  The Gaussian row stays in
-// registers; Sobel clamps in the Gaussian image (G(-1) = G(0), G(W) = G(W-1)).
+// Gaussian5 -> Sobel3 fused (the C5 pipeline).  The Gaussian rows stay in
+// registers; Sobel clamps in the Gaussian image (G(-1) = G(0), G(W) = G(W-1),
+// rows alike).  Input row vy completes Gaussian row gy = vy - 2 and Sobel
+// output row oy = vy - 3.  The last 5 rows of horizontal Gaussian results
+// are a register ring indexed by the compile-time phase U (NWIN = 5); the
+// previous two Gaussian rows shift by register moves.  (Measured on C5: a
+// 15-phase ring of 5 + 3 rows overflowed the instruction cache -- ncu
+// "no_instruction" stalls -- and 4-row + 2-row rings spilled at 128 registers.)  Gaussian rows
+// outside the image, G(-1) and G(H), are replaced by the border row when oy
+// is 0 / H-1.
 struct AppGaussSobel {
   using T = float;
-  static constexpr int V = 8, EW = 4, VR = 3, NIN = 1, NWIN = 1, MINB = 3;
-  float h[5][V + 1];   // horizontal Gaussian of the last 5 input rows: V lane columns + 1 edge column
-  float gs[3][V + 2];  // last 3 Gaussian rows, lane columns -1..V
+  static constexpr int V = 8, EW = 4, VR = 3, NIN = 1, NWIN = 5, MINB = 3;
+  f2 hh[5][V / 2];  // horizontal Gaussian of the last 5 rows, lane columns, pairs
+  float he[5];      // the same for the lane's edge column (xc-1 / xc+V)
+  float gp[V + 2], gq[V + 2];  // Gaussian rows gy-2, gy-1 at lane columns -1 .. V
   __device__ void init(const KParams&) {}
-  __device__ __forceinline__ void push_g(const float (&g)[V + 2]) {
-#pragma unroll
-    for (int k = 0; k < 2; ++k)
-#pragma unroll
-      for (int i = 0; i < V + 2; ++i) gs[k][i] = gs[k + 1][i];
-#pragma unroll
-    for (int i = 0; i < V + 2; ++i) gs[2][i] = g[i];
-  }
   template <int U>
   __device__ __forceinline__ Frag<float, V> row(const Frag<float, V>& c, const Frag<float, EW>& e,
                                                 const Frag<float, V>&, int lane, uint32_t, int vy, int xc,
                                                 const KParams& p) {
+    constexpr int H4 = U % 5, H0 = (U + 1) % 5, H1 = (U + 2) % 5, H2 = (U + 3) % 5, H3 = (U + 4) % 5;  // newest: H4
     float x[V + 4];  // columns xc-2 .. xc+V+1
     ext_row<2, EW, V>(c, e, lane, 0u, x);
-    // edge column (lane 0: xc-1 from e = cols xc-4..xc-1; lane 31: xc+V from e = cols xc+V..xc+V+3)
-    float he;
-    if (lane < 16) {
-      float t[5] = {e.v[1], e.v[2], e.v[3], c.v[0], c.v[1]};
-      he = smooth<2>(t);
-    } else {
-      float t[5] = {c.v[V - 2], c.v[V - 1], e.v[0], e.v[1], e.v[2]};
-      he = smooth<2>(t);
+#pragma unroll
+    for (int j = 0; j < V / 2; ++j) hh[H4][j] = pk2(smooth<2>(x + 2 * j), smooth<2>(x + 2 * j + 1));
+    {  // edge column (lane 0: xc-1 from e = cols xc-4..xc-1; lane 31: xc+V from e = cols xc+V..xc+V+3)
+      float t[5];
+      if (lane < 16) { t[0] = e.v[1]; t[1] = e.v[2]; t[2] = e.v[3]; t[3] = c.v[0]; t[4] = c.v[1]; }
+      else { t[0] = c.v[V - 2]; t[1] = c.v[V - 1]; t[2] = e.v[0]; t[3] = e.v[1]; t[4] = e.v[2]; }
+      he[H4] = smooth<2>(t);
     }
+    // vertical Gaussian over rows gy-2 .. gy+2 (oldest first)
+    float g[V + 2];  // Gaussian row gy at columns xc-1 .. xc+V
+    const f2 sc = splat2(1.f / 256.f);
 #pragma unroll
-    for (int k = 0; k < 4; ++k)
-#pragma unroll
-      for (int i = 0; i <= V; ++i) h[k][i] = h[k + 1][i];
-#pragma unroll
-    for (int i = 0; i < V; ++i) h[4][i] = smooth<2>(x + i);
-    h[4][V] = he;
-    float gv[V + 1];
-#pragma unroll
-    for (int i = 0; i <= V; ++i) {
-      float col[5];
-#pragma unroll
-      for (int k = 0; k < 5; ++k) col[k] = h[k][i];
-      gv[i] = smooth<2>(col) * (1.f / 256.f);
+    for (int j = 0; j < V / 2; ++j) {
+      const f2 a0 = hh[H0][j], a1 = hh[H1][j], a2 = hh[H2][j], a3 = hh[H3][j], a4 = hh[H4][j];
+      up2(mul2(fma2(splat2(6.f), a2, fma2(splat2(4.f), add2(a1, a3), add2(a0, a4))), sc), g[2 * j + 1], g[2 * j + 2]);
     }
-    float g[V + 2];  // Gaussian row gy = vy - 2 at columns xc-1 .. xc+V
-#pragma unroll
-    for (int i = 0; i < V; ++i) g[i + 1] = gv[i];
-    float gl = __shfl_up_sync(FULLMASK, gv[V - 1], 1);
-    float gr = __shfl_down_sync(FULLMASK, gv[0], 1);
-    if (lane == 0) gl = gv[V];
-    if (lane == 31) gr = gv[V];
+    const float gve = fmaf(6.f, he[H2], fmaf(4.f, he[H1] + he[H3], he[H0] + he[H4])) * (1.f / 256.f);
+    float gl = __shfl_up_sync(FULLMASK, g[V], 1);
+    float gright = __shfl_down_sync(FULLMASK, g[1], 1);
+    if (lane == 0) gl = gve;
+    if (lane == 31) gright = gve;
     g[0] = gl;
-    g[V + 1] = gr;
+    g[V + 1] = gright;
     // clamp in the Gaussian image: columns < 0 -> column 0, columns >= W -> column W-1
     if (xc <= 0) g[0] = g[1];
     const int cl = p.W - 1 - xc;  // local index of column W-1
-    if (cl < V) {
-      float gw = g[0];
+    if (cl < V) {  // propagate column W-1 rightwards (prefix selects: no indexed register access)
 #pragma unroll
-      for (int k = 0; k <= V; ++k)
-        if (k == cl + 1) gw = g[k];
-#pragma unroll
-      for (int k = 1; k < V + 2; ++k)
-        if (k > cl + 1) g[k] = gw;
+      for (int k = 1; k < V + 2; ++k) g[k] = k > cl + 1 ? g[k - 1] : g[k];
     }
-    const int gy = vy - 2;  // rows: G(-1) = G(0), G(H) = G(H-1)
-    if (gy == 0) {
-      push_g(g);
-      push_g(g);
-    } else if (gy > 0 && gy < p.Hg) {
-      push_g(g);
-    } else if (gy >= p.Hg) {
-      float last[V + 2];
+    // Sobel3 on Gaussian rows oy-1, oy, oy+1 (oy = vy - 3), clamped at the image's top / bottom
+    const int oy = vy - 3;
+    float t0[V + 2], t1[V + 2], t2[V + 2];
+    const bool top = oy == 0, bot = oy == p.Hg - 1;
 #pragma unroll
-      for (int i = 0; i < V + 2; ++i) last[i] = gs[2][i];
-      push_g(last);
-    } else if (gy < -1) {
-      push_g(g);  // warm-up rows, shifted out before use
+    for (int i = 0; i < V + 2; ++i) {
+      t1[i] = gq[i];
+      t0[i] = top ? gq[i] : gp[i];
+      t2[i] = bot ? gq[i] : g[i];
+      gp[i] = gq[i];
+      gq[i] = g[i];
     }
+    float ev[V + 2];  // vertical derivative per column
+#pragma unroll
+    for (int i = 0; i < V + 2; i += 2) up2(sub2(pk2(t2[i], t2[i + 1]), pk2(t0[i], t0[i + 1])), ev[i], ev[i + 1]);
     Frag<float, V> o;
 #pragma unroll
-    for (int i = 0; i < V; ++i) {
-      const float d0 = gs[0][i + 2] - gs[0][i], d1 = gs[1][i + 2] - gs[1][i], d2 = gs[2][i + 2] - gs[2][i];
-      const float gx = fmaf(2.f, d1, d0 + d2);
-      const float s0 = fmaf(2.f, gs[0][i + 1], gs[0][i] + gs[0][i + 2]);
-      const float s2 = fmaf(2.f, gs[2][i + 1], gs[2][i] + gs[2][i + 2]);
-      const float gyv = s2 - s0;
-      o.v[i] = sqrt_approx(fmaf(gx, gx, gyv * gyv));
+    for (int j = 0; j < V / 2; ++j) {
+      const int i = 2 * j;  // output columns i, i+1 use Gaussian columns i .. i+3 (local -1 offset)
+      const f2 d0 = sub2(pk2(t0[i + 2], t0[i + 3]), pk2(t0[i], t0[i + 1]));
+      const f2 d1 = sub2(pk2(t1[i + 2], t1[i + 3]), pk2(t1[i], t1[i + 1]));
+      const f2 d2 = sub2(pk2(t2[i + 2], t2[i + 3]), pk2(t2[i], t2[i + 1]));
+      const f2 gx = fma2(splat2(2.f), d1, add2(d0, d2));
+      const f2 gy = fma2(splat2(2.f), pk2(ev[i + 1], ev[i + 2]), add2(pk2(ev[i], ev[i + 1]), pk2(ev[i + 2], ev[i + 3])));
+      float m0, m1;
+      up2(fma2(gx, gx, mul2(gy, gy)), m0, m1);
+      o.v[i] = sqrt_approx(m0);
+      o.v[i + 1] = sqrt_approx(m1);
     }
     return o;
   }
