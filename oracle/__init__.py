@@ -30,7 +30,8 @@ METRICS = {"mre": 0, "me": 1, "mae": 2}
 
 class OrcParams(ctypes.Structure):
     _fields_ = [(n, ctypes.c_int) for n in
-                ("app", "W", "H", "radius", "scheme", "num", "den", "recon", "granule", "tile_w", "tile_h")]
+                ("app", "W", "H", "radius", "scheme", "num", "den", "recon", "granule", "tile_w", "tile_h",
+                 "tblock")]
 
 
 def build(force: bool = False) -> str:
@@ -81,9 +82,11 @@ def lib():
     return _lib
 
 
-def params(app="gaussian", W=0, H=0, radius=2, scheme="none", rate=(0, 1), recon="nn", granule=8, tile=(16, 16)):
+def params(app="gaussian", W=0, H=0, radius=2, scheme="none", rate=(0, 1), recon="nn", granule=8, tile=(16, 16),
+           tblock=1):
     num, den = rate
-    return OrcParams(APPS[app], W, H, radius, SCHEMES[scheme], num, den, RECONS[recon], granule, tile[0], tile[1])
+    return OrcParams(APPS[app], W, H, radius, SCHEMES[scheme], num, den, RECONS[recon], granule, tile[0], tile[1],
+                     tblock)
 
 
 def _ptr(a: np.ndarray):

@@ -328,7 +328,8 @@ int orc_run_pixel_u8(const orc_params* p, const uint8_t* in, int x, int y) {
  * with clamped neighbours.  Reading R13: Rodinia's constants with the cell
  * size of the 1024 x 1024 chip fixed for every grid size (the literal
  * constants are unstable beyond n ~ 1386).  R14: T and P are both perforated
- * and rebuilt every step.                                                  */
+ * and rebuilt every step.  R19: with temporal blocking (tblock > 1) T is
+ * perforated at every tblock-th step only.                                 */
 void orc_hotspot_coeffs(double* step_div_cap, double* rx_1, double* ry_1, double* rz_1, double* amb) {
   const double t_chip = 0.0005, chip = 0.016;
   const double gw = chip / 1024.0, gh = chip / 1024.0;
@@ -362,10 +363,16 @@ static void hotspot_window(const orc_params* p, double* T, const float* P, int o
   for (int y = 0; y < h; ++y)
     for (int x = 0; x < w; ++x) Pr[(long long)y * w + x] = recon_f(&vp, x, y);
   view_t vt = vp; vt.f32 = NULL;
+  const int tb = p->tblock > 1 ? p->tblock : 1;
   for (int it = 0; it < iters; ++it) {
     vt.f64 = T;
+    /* R19 (temporal blocking): a kernel that keeps T on chip
+     * for tb steps loads it from memory -- perforated, then rebuilt -- only
+     * at the first of them; the other steps read the full on-chip T. */
+    const int perforate = (it % tb) == 0;
     for (int y = 0; y < h; ++y)
-      for (int x = 0; x < w; ++x) Tr[(long long)y * w + x] = recon_f(&vt, x, y);
+      for (int x = 0; x < w; ++x)
+        Tr[(long long)y * w + x] = perforate ? recon_f(&vt, x, y) : T[(long long)y * w + x];
     for (int y = 0; y < h; ++y)
       for (int x = 0; x < w; ++x) {
         const double tc = Tr[(long long)y * w + x];

@@ -34,6 +34,8 @@ typedef struct {
   int recon;
   int granule;          /* G: pixels per column/checker cell (>= 1) */
   int tile_w, tile_h;   /* STENCIL1: work-group tile of output pixels */
+  int tblock;           /* Hotspot temporal blocking (R19): T is perforated and rebuilt
+                           only at steps it with it % tblock == 0 (<= 1: every step) */
 } orc_params;
 
 /* Step 1 -- perforation mask (1 = loaded / kept, 0 = skipped). */
@@ -53,7 +55,8 @@ double orc_run_pixel_f32(const orc_params* p, const float* in, int x, int y);
 int orc_run_pixel_u8(const orc_params* p, const uint8_t* in, int x, int y);
 
 /* Hotspot (Rodinia 2D transient thermal stencil), iters steps; T and P both
- * perforated and rebuilt every step. */
+ * perforated and rebuilt every step (every tblock-th step for T when
+ * tblock > 1; P is static, so its rebuild is the same at every step). */
 void orc_hotspot_coeffs(double* step_div_cap, double* rx_1, double* ry_1, double* rz_1, double* amb);
 void orc_hotspot_run(const orc_params* p, const float* T0, const float* P, int iters, double* Tout);
 /* iters steps on a window of the global grid (origin ox, oy; w x h); T is

@@ -501,3 +501,96 @@ def test_p13_stencil1_paper_claims():
     e_s1 = oracle.error("mre", ex, oracle.run(p, img))[0]
     e_r1 = oracle.error("mre", ex, oracle.run(P("gaussian", W, H, 1, "row", (1, 2), "nn"), img))[0]
     assert e_s1 < 0.01 and e_s1 < e_r1
+
+
+# --------------------------------------------------------------------------
+# P14: Hotspot temporal blocking (R19): with tblock
+# = p, T is perforated and rebuilt only at steps it % p == 0 -- the steps a
+# p-step-per-launch kernel loads T from memory; the others read on-chip T.
+def _np_hotspot(T0, P0, iters, den, num, recon, tblock):
+    """independent numpy formulation: explicit kept-row list, np.pad(edge)
+    clamp, Rodinia update in fp64"""
+    sdc, rx1, ry1, rz1, amb = oracle.hotspot_coeffs()
+    H, W = T0.shape
+    keep_one = num == den - 1
+    kept = [y for y in range(H) if (y % den == 0 if keep_one else y % den != den - 1)]
+
+    def rebuild(A):
+        R = A.copy()
+        for y in range(H):
+            if y in kept:
+                continue
+            lo = [k for k in kept if k < y]
+            hi = [k for k in kept if k > y]
+            a, b = (lo[-1] if lo else None), (hi[0] if hi else None)
+            if recon == "li" and a is not None and b is not None:
+                R[y] = (A[a] * (b - y) + A[b] * (y - a)) / (b - a)
+            elif b is None or (a is not None and y - a <= b - y):
+                R[y] = A[a]
+            else:
+                R[y] = A[b]
+        return R
+
+    T = T0.astype(np.float64)
+    Pr = rebuild(P0.astype(np.float64))
+    for it in range(iters):
+        Tr = rebuild(T) if it % tblock == 0 else T
+        Q = np.pad(Tr, 1, mode="edge")
+        lap_y = Q[2:, 1:-1] + Q[:-2, 1:-1] - 2 * Tr
+        lap_x = Q[1:-1, 2:] + Q[1:-1, :-2] - 2 * Tr
+        T = Tr + sdc * (Pr + lap_y * ry1 + lap_x * rx1 + (amb - Tr) * rz1)
+    return T
+
+
+@pytest.mark.parametrize("rate,recon", [((1, 2), "li"), ((1, 2), "nn"), ((3, 4), "li"), ((1, 3), "nn")])
+@pytest.mark.parametrize("tblock", [1, 2, 3, 8])
+def test_p14_hotspot_tblock_vs_numpy(rate, recon, tblock):
+    W, H, iters = 9, 13, 7
+    T, Pw = synth.hotspot(11, W, H)
+    p = oracle.params("hotspot", W, H, 1, "row", rate, recon, 8, tblock=tblock)
+    got = oracle.hotspot(p, T, Pw, iters)
+    want = _np_hotspot(T, Pw, iters, rate[1], rate[0], recon, tblock)
+    assert np.allclose(got, want, rtol=1e-13, atol=0)
+
+
+def test_p14_hotspot_tblock_invariants():
+    sdc, rx1, ry1, rz1, amb = oracle.hotspot_coeffs()
+    W, H = 12, 10
+    T, Pw = synth.hotspot(5, W, H)
+    base = oracle.hotspot(oracle.params("hotspot", W, H, 1, "row", (1, 2), "li", 8), T, Pw, 6)
+    # tblock 1 (and 0) is the per-step definition
+    for tb in (0, 1):
+        p = oracle.params("hotspot", W, H, 1, "row", (1, 2), "li", 8, tblock=tb)
+        assert np.array_equal(oracle.hotspot(p, T, Pw, 6), base)
+    # rate 0 is exact whatever tblock
+    ex = oracle.hotspot(oracle.params("hotspot", W, H, 1), T, Pw, 6)
+    assert np.array_equal(oracle.hotspot(oracle.params("hotspot", W, H, 1, tblock=3), T, Pw, 6), ex)
+    # fixed point and the uniform closed-form decay hold for any tblock
+    T0, P0 = 330.0, 0.005
+    Tu = np.full((H, W), T0, dtype=np.float32)
+    Pu = np.full((H, W), P0, dtype=np.float32)
+    Tstar = amb + np.float64(np.float32(P0)) / rz1
+    for tb in (2, 5):
+        p = oracle.params("hotspot", W, H, 1, "row", (3, 4), "li", 8, tblock=tb)
+        assert np.array_equal(oracle.hotspot(p, np.full((H, W), 80.0, np.float32), np.zeros((H, W), np.float32), 7),
+                              np.full((H, W), 80.0))
+        assert np.allclose(oracle.hotspot(p, Tu, Pu, 9), Tstar + (T0 - Tstar) * (1 - sdc * rz1) ** 9, rtol=1e-12)
+    # tblock >= iters perforates T once: equals 1 perforated step then exact steps
+    p1 = oracle.params("hotspot", W, H, 1, "row", (1, 2), "li", 8)
+    T64 = T.astype(np.float64)
+    oracle.hotspot_window(p1, T64, Pw, 0, 0, 1)
+    oracle.hotspot_window(oracle.params("hotspot", W, H, 1, "none", (0, 1), "nn", 8), T64,
+                          oracle.reconstruct(p1, Pw).astype(np.float32), 0, 0, 5)
+    got = oracle.hotspot(oracle.params("hotspot", W, H, 1, "row", (1, 2), "li", 8, tblock=6), T, Pw, 6)
+    assert np.allclose(got, T64, rtol=1e-13)
+
+
+def test_p14_hotspot_tblock_perforates_less():
+    """fewer perforated loads -> error against the exact run does not grow
+    (synthetic C4-like grid, 24 steps)"""
+    W, H = 96, 64
+    T, Pw = synth.hotspot(synth.SEED_C4, W, H)
+    ex = oracle.hotspot(oracle.params("hotspot", W, H, 1), T, Pw, 24)
+    errs = [oracle.error("mre", ex, oracle.hotspot(oracle.params("hotspot", W, H, 1, "row", (1, 2), "li", 8,
+                                                                 tblock=tb), T, Pw, 24))[0] for tb in (1, 4, 24)]
+    assert errs[0] > errs[1] > errs[2] > 0
