@@ -300,6 +300,8 @@ def main():
     ap.add_argument("--no-variants", action="store_true")
     ap.add_argument("--no-cpu", action="store_true")
     ap.add_argument("--batch", type=int, default=0)
+    ap.add_argument("--tblock", type=int, default=1,
+                    help="C4 only: Hotspot steps per launch (temporal blocking, DESIGN.md R19); 1 = per-step")
     args = ap.parse_args()
     args.warmup = max(args.warmup, 3)
 
@@ -500,7 +502,7 @@ def bench_hotspot(args, cfg, ws, rank, local, stream, peak, peak_src):
     P = torch.empty((h, W), device="cuda")
     synth.hotspot_band_device(cfg["seed"], W, Hg, y0, h, T.data_ptr(), P.data_ptr(), stream.cuda_stream)
     out = torch.empty_like(T)
-    keys = dict(iters=iters)
+    keys = dict(iters=iters, tblock=args.tblock)
     if ws > 1:
         keys.update(global_h=Hg, band_y0=y0)
     plan = kp.Plan("hotspot", W, h, 1, cfg["scheme"], cfg["rate"], cfg["recon"], **keys)
@@ -534,6 +536,24 @@ def bench_hotspot(args, cfg, ws, rank, local, stream, peak, peak_src):
     cells = W * Hg * iters
     algo_b = bytes_per_px("hotspot", cfg["scheme"], cfg["rate"]) * W * h * iters
     achieved = algo_b / (ms * 1e-3) / 1e9
+    # NEXT-3 temporal blocking (single band only): TBLOCK steps per launch, T
+    # perforated once per launch (R19) -- reported next to the
+    # per-step headline, never in its place
+    tblock = []
+    if ws == 1 and not args.no_variants:
+        for tb in (2, 4, 8):
+            for sch, rt, rc in ((cfg["scheme"], cfg["rate"], cfg["recon"]), ("none", (0, 1), "nn")):
+                q = kp.Plan("hotspot", W, h, 1, sch, rt, rc, iters=iters, tblock=tb)
+                o2 = torch.empty_like(T)
+                ms_tb = time_kernel(lambda: q.hotspot(T, P, o2, stream), stream, 3, 1)
+                e_tb, _ = q.error(out_ex, o2, stream)
+                tblock.append({"tblock": tb, "scheme": sch, "rate": list(rt), "recon": rc, "ms": ms_tb,
+                               "mcell_s": cells / (ms_tb * 1e-3) / 1e6, "speedup_vs_exact_per_step": ms_ex / ms_tb,
+                               "error_vs_exact_per_step": e_tb,
+                               # kept T + P read and T' written once per launch of tb steps
+                               "algorithmic_gbs": bytes_per_px("hotspot", sch, rt) * W * h * iters / tb
+                               / (ms_tb * 1e-3) / 1e9})
+                q.close()
     scratch = torch.empty((2, h, W), device="cuda")
     pmix = mixed_peak_gbs(scratch.data_ptr(), out_ex.data_ptr(), W * h * 4, cfg["scheme"], cfg["rate"], 128,
                           n_in=2, stream=stream.cuda_stream, pitch_bytes=W * 4)
@@ -541,13 +561,15 @@ def bench_hotspot(args, cfg, ws, rank, local, stream, peak, peak_src):
     return {"metric": METRIC, "value": cells / (ms * 1e-3) / 1e6, "unit": "Mcell-updates/s", "n_gpus": ws,
             "steps": args.steps, "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True,
             "scaling": "strong", "vs_baseline": None, "dtype": "f32", "data": "synthetic",
-            "config": {"workload": cfg["workload"], "bands": ws, "halo": "NCCL send/recv per step" if ws > 1
-                       else "none"},
+            "config": {"workload": cfg["workload"] + (f", temporal blocking {args.tblock} steps/launch"
+                                                      if args.tblock > 1 else ""),
+                       "bands": ws, "tblock": args.tblock,
+                       "halo": ("NCCL send/recv per launch" if ws > 1 else "none")},
             "speedup_vs_exact": ms_ex / ms, "error": {"metric": "mre", "value": mre, "count": cnt},
             "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
                          "frac": achieved / peak, "traffic": None, "peak_source": peak_src,
                          "peak_mix": pmix, "frac_mix": achieved / pmix if pmix else None},
-            "clocks": clk.summary(), "gpu_launches": args.steps * iters}
+            "clocks": clk.summary(), "gpu_launches": args.steps * (-(-iters // args.tblock)), "temporal_blocking": tblock}
 
 
 if __name__ == "__main__":

@@ -102,7 +102,11 @@ enum {
   PERF_KEY_HALO_ROWS = 11,     /* read-only: rows a Hotspot band exchanges with each neighbour per step */
   PERF_KEY_TILE1_W = 12,       /* STENCIL1 tile width: power of two, 16..256 (fp32) / 16..512 (u8); default 16 */
   PERF_KEY_TILE1_H = 13,       /* STENCIL1 tile height, 1..1024; default 16 */
-  PERF_KEY_PRODUCER = 14       /* 0 auto = 1 dedicated producer warp; 2 bulk rows issued by consumer warp 0 */
+  PERF_KEY_PRODUCER = 14,      /* 0 auto = 1 dedicated producer warp; 2 bulk rows issued by consumer warp 0 */
+  PERF_KEY_TBLOCK = 15         /* Hotspot temporal blocking: steps per launch, 1..8 (default 1).  CHANGES
+                                  RESULTS: T is loaded (perforated, rebuilt) once per launch and the other
+                                  steps of the launch read on-chip T (R19).
+                                  NONE / ROW schemes; single-band plans */
 };
 
 /* Create a plan.  Validates: W, H >= 1; radius allowed for the app (Gaussian,
@@ -126,7 +130,10 @@ perf_status perf_run_host(perf_plan_t plan, const void* host_in, void* host_out,
 
 /* ITERS Hotspot steps on device buffers of W * H floats (a band of H rows
  * starting at global row BAND_Y0 of a GLOBAL_H-row grid when sharded).  T and
- * P are both perforated and rebuilt every step.  temp_in is not modified. */
+ * P are both perforated and rebuilt every step -- every TBLOCK-th step for T
+ * when TBLOCK > 1 (one launch per TBLOCK steps, T kept in shared memory in
+ * between; PERF_ERR_UNSUPPORTED for COL/CHECKER or banded plans).  temp_in is
+ * not modified. */
 perf_status perf_run_hotspot(perf_plan_t plan, const float* temp_in, const float* power, float* temp_out,
                              void* stream);
 

@@ -12,6 +12,7 @@
 #include <vector>
 
 #include "../../include/kperf.h"
+#include "hotspot_tb.cuh"
 #include "kernel.cuh"
 
 namespace kp {
@@ -48,7 +49,7 @@ struct perf_plan_s {
   int app, W, H, radius, scheme, recon;
   perf_rate rate;
   long long batch = 1, iters = 1, granule_bytes = 128, global_h = -1, band_y0 = 0, tile_w = kp::kNCW, tile_h = 0,
-            metric = 0, loader = 0, ring = 0, tile1_w = 16, tile1_h = 16, producer = 0;
+            metric = 0, loader = 0, ring = 0, tile1_w = 16, tile1_h = 16, producer = 0, tblock = 1;
   double* d_err = nullptr;
   float* d_tmp = nullptr;
   size_t tmp_elems = 0;
@@ -71,6 +72,21 @@ static int log2i(int v) {
   int l = 0;
   while ((1 << l) < v) ++l;
   return l;
+}
+
+// Rodinia Hotspot coefficients, cell size of the 1024 x 1024 chip (R13)
+static void hotspot_coeffs(float& sdc, float& rx1, float& ry1, float& rz1, float& amb) {
+  const double t_chip = 0.0005, chip = 0.016, gw = chip / 1024.0, gh = chip / 1024.0;
+  const double cap = 0.5 * 1.75e6 * t_chip * gw * gh;
+  const double rx = gw / (2.0 * 100.0 * t_chip * gh), ry = gh / (2.0 * 100.0 * t_chip * gw);
+  const double rz = t_chip / (100.0 * gh * gw);
+  const double max_slope = 3.0e6 / (0.5 * t_chip * 1.75e6);
+  const double step = 0.001 / max_slope;
+  sdc = (float)(step / cap);
+  rx1 = (float)(1.0 / rx);
+  ry1 = (float)(1.0 / ry);
+  rz1 = (float)(1.0 / rz);
+  amb = 80.0f;
 }
 
 // Launch geometry for rows [y_begin, y_end) of `frames` frames.
@@ -162,20 +178,7 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   const long long g = (long long)k.n_strips * k.n_segs * frames;
   if (g <= 0 || g > 0x7FFFFFFFLL) return fail(PERF_ERR_INVALID_ARG, "grid size out of range");
   grid = (unsigned)g;
-  // Rodinia Hotspot coefficients, cell size of the 1024 x 1024 chip (R13)
-  {
-    const double t_chip = 0.0005, chip = 0.016, gw = chip / 1024.0, gh = chip / 1024.0;
-    const double cap = 0.5 * 1.75e6 * t_chip * gw * gh;
-    const double rx = gw / (2.0 * 100.0 * t_chip * gh), ry = gh / (2.0 * 100.0 * t_chip * gw);
-    const double rz = t_chip / (100.0 * gh * gw);
-    const double max_slope = 3.0e6 / (0.5 * t_chip * 1.75e6);
-    const double step = 0.001 / max_slope;
-    k.sdc = (float)(step / cap);
-    k.rx1 = (float)(1.0 / rx);
-    k.ry1 = (float)(1.0 / ry);
-    k.rz1 = (float)(1.0 / rz);
-    k.amb = 80.0f;
-  }
+  hotspot_coeffs(k.sdc, k.rx1, k.ry1, k.rz1, k.amb);
   return PERF_OK;
 }
 
@@ -198,9 +201,38 @@ static cudaError_t dispatch(const perf_plan_s* P, const KParams& k, unsigned gri
 }
 
 static int band_halo(const perf_plan_s* p) {
-  // stencil radius 1 + distance to the loaded rows a rebuilt row reads
+  // stencil radius 1 per step of a launch (TBLOCK steps under temporal
+  // blocking) + distance to the loaded rows a rebuilt row reads
   const bool vertical = p->rate.num > 0 && (p->scheme == PERF_SCHEME_ROW || p->scheme == PERF_SCHEME_CHECKER);
-  return 1 + (vertical ? p->rate.den : 0);
+  return (int)p->tblock + (vertical ? p->rate.den : 0);
+}
+
+// temporally blocked Hotspot launch parameters (hotspot_tb.cu) for a plan
+static kp::TBParams tb_params(const perf_plan_s* p, const float* T, const float* P, float* out) {
+  kp::TBParams q;
+  std::memset(&q, 0, sizeof q);
+  q.T = T;
+  q.P = P;
+  q.out = out;
+  q.W = p->W;
+  q.Hg = p->global_h > 0 ? (int)p->global_h : p->H;
+  q.avail1 = q.Hg;
+  q.y_end = q.Hg;
+  q.row_scheme = (p->rate.num > 0 && p->scheme == PERF_SCHEME_ROW) ? 1 : 0;
+  q.den = q.row_scheme ? p->rate.den : 1;
+  q.keep_one = q.row_scheme && p->rate.num == p->rate.den - 1;
+  q.li = p->recon == PERF_RECON_LINEAR;
+  q.apron = q.row_scheme ? q.den - 1 : 0;
+  q.vec = (p->W % 4 == 0) && (((reinterpret_cast<uintptr_t>(T) | reinterpret_cast<uintptr_t>(P) |
+                                 reinterpret_cast<uintptr_t>(out)) & 15) == 0);
+  float sdc, rx1, ry1, rz1, amb;  // regrouped Rodinia coefficients from the same fp32 constants
+  hotspot_coeffs(sdc, rx1, ry1, rz1, amb);
+  q.sdc = sdc;
+  q.cx = (float)((double)sdc * rx1);
+  q.cy = (float)((double)sdc * ry1);
+  q.c0 = (float)(1.0 - 2.0 * (double)sdc * rx1 - 2.0 * (double)sdc * ry1 - (double)sdc * rz1);
+  q.pamb = (float)((double)sdc * amb * rz1);
+  return q;
 }
 
 
@@ -311,6 +343,10 @@ perf_status perf_plan_set(perf_plan_t p, int key, long long v) {
       if (v < 0 || v > 2) return fail(PERF_ERR_INVALID_ARG, "PRODUCER must be 0 (auto), 1 (dedicated) or 2 (inline)");
       p->producer = v;
       return PERF_OK;
+    case PERF_KEY_TBLOCK:
+      if (v < 1 || v > 8) return fail(PERF_ERR_INVALID_ARG, "TBLOCK must be in [1, 8]");
+      p->tblock = v;
+      return PERF_OK;
   }
   return fail(PERF_ERR_INVALID_ARG, "unknown key");
 }
@@ -332,6 +368,7 @@ perf_status perf_plan_get(perf_plan_t p, int key, long long* v) {
     case PERF_KEY_TILE1_W: *v = p->tile1_w; return PERF_OK;
     case PERF_KEY_TILE1_H: *v = p->tile1_h; return PERF_OK;
     case PERF_KEY_PRODUCER: *v = p->producer; return PERF_OK;
+    case PERF_KEY_TBLOCK: *v = p->tblock; return PERF_OK;
   }
   return fail(PERF_ERR_INVALID_ARG, "unknown key");
 }
@@ -392,8 +429,20 @@ static perf_status band_alloc(perf_plan_s* p) {
 }
 
 // one step of a band: rows [y0, y0+h) of buffer `src` (with halos filled) -> `dst`
-static perf_status band_step(perf_plan_s* p, const float* src, float* dst, cudaStream_t s) {
+static perf_status band_step(perf_plan_s* p, const float* src, float* dst, int steps, cudaStream_t s) {
   const int Hg = (int)p->global_h, y0 = (int)p->band_y0, h = p->H, hb = p->band.hb;
+  if (p->tblock > 1) {  // `steps` steps in one temporally blocked launch
+    kp::TBParams q = tb_params(p, src, p->band.pbuf, dst);
+    q.in_row0 = q.out_row0 = y0 - hb;
+    q.avail0 = std::max(0, y0 - hb);
+    q.avail1 = std::min(Hg, y0 + h + hb);
+    q.y_begin = y0;
+    q.y_end = y0 + h;
+    q.steps = steps;
+    cudaError_t e = kp::launch_hotspot_tb(q, s);
+    if (e != cudaSuccess) return cuda_fail(e, "hotspot band launch (temporal blocking)");
+    return PERF_OK;
+  }
   KParams k;
   unsigned grid;
   size_t smem;
@@ -436,6 +485,31 @@ perf_status perf_run_hotspot(perf_plan_t p, const float* temp_in, const float* p
     CK(cudaMemcpyAsync(temp_out, temp_in, n * sizeof(float), cudaMemcpyDeviceToDevice, s));
     return PERF_OK;
   }
+  if (p->tblock > 1) {
+    const bool exact = p->rate.num == 0 || p->scheme == PERF_SCHEME_NONE;
+    if (!exact && p->scheme != PERF_SCHEME_ROW) return fail(PERF_ERR_UNSUPPORTED, "TBLOCK > 1 needs the NONE or ROW scheme");
+  }
+  if (!banded && p->tblock > 1) {  // temporal blocking: one launch per TBLOCK steps
+    const long long tb = p->tblock, launches = (p->iters + tb - 1) / tb;
+    if (launches > 1 && p->tmp_elems < (size_t)n) {
+      if (p->d_tmp) cudaFree(p->d_tmp);
+      p->d_tmp = nullptr;
+      if (cudaMalloc(&p->d_tmp, n * sizeof(float)) != cudaSuccess) return fail(PERF_ERR_OOM, "tmp allocation");
+      p->tmp_elems = n;
+    }
+    const float* src = temp_in;
+    for (long long l = 0; l < launches; ++l) {
+      float* dst = ((launches - 1 - l) % 2 == 0) ? temp_out : p->d_tmp;
+      kp::TBParams q = tb_params(p, src, power, dst);
+      q.vec = q.vec && ((reinterpret_cast<uintptr_t>(temp_in) | reinterpret_cast<uintptr_t>(temp_out) |
+                         reinterpret_cast<uintptr_t>(p->d_tmp)) & 15) == 0;
+      q.steps = (int)std::min(tb, p->iters - l * tb);
+      cudaError_t e = kp::launch_hotspot_tb(q, s);
+      if (e != cudaSuccess) return cuda_fail(e, "hotspot (temporal blocking) launch");
+      src = dst;
+    }
+    return PERF_OK;
+  }
   if (!banded) {
     if (p->iters > 1 && p->tmp_elems < (size_t)n) {
       if (p->d_tmp) cudaFree(p->d_tmp);
@@ -469,9 +543,10 @@ perf_status perf_run_hotspot(perf_plan_t p, const float* temp_in, const float* p
   CK(cudaMemcpyAsync(p->band.pbuf + hb * W, power, n * sizeof(float), cudaMemcpyDeviceToDevice, s));
   if ((st = band_exchange_nccl(p, p->band.pbuf, s)) != PERF_OK) return st;
   int cur = 0;
-  for (long long i = 0; i < p->iters; ++i) {
+  for (long long i = 0; i < p->iters; i += p->tblock) {  // one halo exchange + launch per TBLOCK steps
     if ((st = band_exchange_nccl(p, p->band.buf[cur], s)) != PERF_OK) return st;
-    if ((st = band_step(p, p->band.buf[cur], p->band.buf[cur ^ 1], s)) != PERF_OK) return st;
+    const int steps = (int)std::min(p->tblock, p->iters - i);
+    if ((st = band_step(p, p->band.buf[cur], p->band.buf[cur ^ 1], steps, s)) != PERF_OK) return st;
     cur ^= 1;
   }
   CK(cudaMemcpyAsync(temp_out, p->band.buf[cur] + hb * W, n * sizeof(float), cudaMemcpyDeviceToDevice, s));
@@ -489,8 +564,10 @@ perf_status perf_run_hotspot_bands_local(perf_plan_t* plans, int nb, const float
   const long long iters = plans[0]->iters;
   for (int b = 0; b < nb; ++b) {
     perf_plan_s* p = plans[b];
-    if (!p || p->app != PERF_APP_HOTSPOT || (size_t)p->W != W || p->iters != iters)
-      return fail(PERF_ERR_INVALID_ARG, "band plans must be Hotspot plans of one grid");
+    if (!p || p->app != PERF_APP_HOTSPOT || (size_t)p->W != W || p->iters != iters || p->tblock != plans[0]->tblock)
+      return fail(PERF_ERR_INVALID_ARG, "band plans must be Hotspot plans of one grid (same ITERS, TBLOCK)");
+    if (p->tblock > 1 && p->rate.num > 0 && p->scheme != PERF_SCHEME_ROW && p->scheme != PERF_SCHEME_NONE)
+      return fail(PERF_ERR_UNSUPPORTED, "TBLOCK > 1 needs the NONE or ROW scheme");
     if (b > 0 && p->band_y0 != plans[b - 1]->band_y0 + plans[b - 1]->H)
       return fail(PERF_ERR_INVALID_ARG, "bands must be consecutive");
     perf_status st = band_alloc(p);
@@ -523,10 +600,13 @@ perf_status perf_run_hotspot_bands_local(perf_plan_t* plans, int nb, const float
   perf_status st = exchange(0, true);
   if (st != PERF_OK) return st;
   int cur = 0;
-  for (long long i = 0; i < iters; ++i) {
+  const long long tb = plans[0]->tblock;
+  for (long long i = 0; i < iters; i += tb) {
     if ((st = exchange(cur, false)) != PERF_OK) return st;
+    const int steps = (int)std::min(tb, iters - i);
     for (int b = 0; b < nb; ++b)
-      if ((st = band_step(plans[b], plans[b]->band.buf[cur], plans[b]->band.buf[cur ^ 1], s)) != PERF_OK) return st;
+      if ((st = band_step(plans[b], plans[b]->band.buf[cur], plans[b]->band.buf[cur ^ 1], steps, s)) != PERF_OK)
+        return st;
     cur ^= 1;
   }
   for (int b = 0; b < nb; ++b) {

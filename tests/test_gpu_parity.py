@@ -259,13 +259,17 @@ def test_hotspot_parity(scheme, rate, recon, iters):
 @pytest.mark.parametrize("scheme,rate,recon", [("none", (0, 1), "nn"), ("row", (1, 2), "li"),
                                                ("row", (3, 4), "nn"), ("checker", (1, 2), "li")])
 @pytest.mark.parametrize("nb", [2, 3, 4])
-def test_hotspot_bands_equal_whole_grid(scheme, rate, recon, nb):
-    """Sharding semantics: row bands with halo exchange == one grid, bit for bit."""
+@pytest.mark.parametrize("tb", [1, 4])
+def test_hotspot_bands_equal_whole_grid(scheme, rate, recon, nb, tb):
+    """Sharding semantics: row bands with halo exchange == one grid, bit for bit
+    (tb > 1: temporally blocked launches, one halo exchange per launch)."""
+    if tb > 1 and scheme == "checker":
+        pytest.skip("temporal blocking: NONE / ROW schemes")
     W, H, iters = 640, 200, 9
     T, P = synth.hotspot(7, W, H)
     Td, Pd = torch.from_numpy(T).cuda(), torch.from_numpy(P).cuda()
     whole = torch.empty_like(Td)
-    with kp.Plan("hotspot", W, H, 1, scheme, rate, recon, iters=iters) as p:
+    with kp.Plan("hotspot", W, H, 1, scheme, rate, recon, iters=iters, tblock=tb) as p:
         p.hotspot(Td, Pd, whole)
     cuts = np.linspace(0, H, nb + 1).astype(int)
     cuts[1:-1] += 3  # uneven bands
@@ -273,13 +277,85 @@ def test_hotspot_bands_equal_whole_grid(scheme, rate, recon, nb):
     for b in range(nb):
         h = int(cuts[b + 1] - cuts[b])
         plans.append(kp.Plan("hotspot", W, h, 1, scheme, rate, recon, iters=iters, global_h=H,
-                             band_y0=int(cuts[b])))
+                             band_y0=int(cuts[b]), tblock=tb))
     banded = torch.empty_like(Td)
     kp.perf_run_hotspot_bands_local([q.handle for q in plans], Td, Pd, banded)
     torch.cuda.synchronize()
     assert torch.equal(banded, whole)
     for q in plans:
         q.close()
+
+
+# ---------------------------------------------------------------------------
+# Hotspot temporal blocking (R19): TBLOCK steps per
+# launch, T perforated at the first step of each launch -- oracle `tblock`
+@pytest.mark.parametrize("scheme,rate,recon", [("none", (0, 1), "nn"), ("row", (1, 2), "li"),
+                                               ("row", (1, 2), "nn"), ("row", (3, 4), "li"),
+                                               ("row", (1, 3), "nn"), ("row", (7, 8), "li")])
+@pytest.mark.parametrize("tb,iters", [(2, 1), (2, 7), (4, 16), (8, 13), (3, 9)])
+def test_hotspot_tblock_parity(scheme, rate, recon, tb, iters):
+    W, H = 1100, 260  # several 144..156-column x 32..44-row tiles, ragged tails
+    T, P = synth.hotspot(synth.SEED_C4, W, H)
+    Td, Pd = torch.from_numpy(T).cuda(), torch.from_numpy(P).cuda()
+    out = torch.empty_like(Td)
+    with kp.Plan("hotspot", W, H, 1, scheme, rate, recon, iters=iters, tblock=tb) as p:
+        p.hotspot(Td, Pd, out)
+        torch.cuda.synchronize()
+    want = oracle.hotspot(oracle.params("hotspot", W, H, 1, scheme, rate, recon, 8, tblock=tb), T, P, iters)
+    assert_close("hotspot", 1, out.cpu().numpy(), want)
+    assert np.array_equal(Td.cpu().numpy(), T)
+
+
+@pytest.mark.parametrize("shape", [(1, 1), (5, 3), (7, 2), (101, 13), (1101, 97), (160, 48), (144, 32)])
+@pytest.mark.parametrize("tb", [2, 8])
+def test_hotspot_tblock_ragged(shape, tb):
+    W, H = shape  # W % 4 != 0 takes the scalar loader
+    T, P = synth.hotspot(3, W, H)
+    Td, Pd = torch.from_numpy(T).cuda(), torch.from_numpy(P).cuda()
+    out = torch.empty_like(Td)
+    with kp.Plan("hotspot", W, H, 1, "row", (1, 2), "li", iters=11, tblock=tb) as p:
+        p.hotspot(Td, Pd, out)
+        torch.cuda.synchronize()
+    want = oracle.hotspot(oracle.params("hotspot", W, H, 1, "row", (1, 2), "li", 8, tblock=tb), T, P, 11)
+    assert_close("hotspot", 1, out.cpu().numpy(), want)
+
+
+def test_hotspot_tblock1_is_per_step():
+    W, H = 300, 70
+    T, P = synth.hotspot(9, W, H)
+    Td, Pd = torch.from_numpy(T).cuda(), torch.from_numpy(P).cuda()
+    a, b = torch.empty_like(Td), torch.empty_like(Td)
+    with kp.Plan("hotspot", W, H, 1, "row", (1, 2), "li", iters=5) as p:
+        p.hotspot(Td, Pd, a)
+    with kp.Plan("hotspot", W, H, 1, "row", (1, 2), "li", iters=5, tblock=1) as p:
+        p.hotspot(Td, Pd, b)
+    torch.cuda.synchronize()
+    assert torch.equal(a, b)
+    with pytest.raises(RuntimeError):
+        with kp.Plan("hotspot", W, H, 1, "col", (1, 2), "li", iters=5, tblock=2) as p:
+            p.hotspot(Td, Pd, b)
+
+
+def test_c4_hotspot_tblock_cone_sampled():
+    """4096^2 x 40 steps with TBLOCK 4 (the bench's C4 temporal-blocking
+    variant); oracle on the dependency cones of a few patches"""
+    W = H = 4096
+    iters, tb = 40, 4
+    T = torch.empty((H, W), device="cuda")
+    P = torch.empty((H, W), device="cuda")
+    synth.hotspot_device(synth.SEED_C4, W, H, T.data_ptr(), P.data_ptr())
+    out = torch.empty_like(T)
+    with kp.Plan("hotspot", W, H, 1, "row", (1, 2), "li", iters=iters, tblock=tb) as p:
+        p.hotspot(T, P, out)
+    torch.cuda.synchronize()
+    Th, Ph = T.cpu().numpy(), P.cpu().numpy()
+    o = out.cpu().numpy()
+    prm = oracle.params("hotspot", W, H, 1, "row", (1, 2), "li", tblock=tb)
+    for x0, y0 in [(0, 0), (2000, 1500), (4090, 4090), (151, 39), (777, 4093)]:
+        w = min(6, W - x0)
+        h = min(3, H - y0)
+        want = oracle.hotspot_rect(prm, Th, Ph, iters, x0, y0, w, h)
+        assert_close("hotspot", 1, o[y0:y0 + h, x0:x0 + w], want)
 
 
 # ---------------------------------------------------------------------------

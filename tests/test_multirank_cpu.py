@@ -4,7 +4,8 @@ Each rank owns the row band kp.band_cuts(H, n)[rank:rank+2] with halo_rows =
 perf_plan_get(plan, "halo_rows") rows on each side (queried from libkperf,
 no GPU needed) and, every step, exchanges halos with the same choreography as
 kperf.cu's NCCL path (my first halo rows -> rank-1's bottom halo, my last halo
-rows -> rank+1's top halo), then advances its window one step with the
+rows -> rank+1's top halo), then advances its window one launch (1 step, or
+TBLOCK steps under temporal blocking) with the
 oracle's windowed Hotspot (global-coordinate mask).  The gathered bands must
 equal the whole-grid oracle bit for bit: this pins the band partition, the
 halo size and the exchange pattern the GPU path uses.
@@ -31,7 +32,7 @@ def _free_port():
         return s.getsockname()[1]
 
 
-def _worker(rank, n, port, scheme, rate, recon, q):
+def _worker(rank, n, port, scheme, rate, recon, q, tb=1):
     os.environ["MASTER_ADDR"] = "127.0.0.1"
     os.environ["MASTER_PORT"] = str(port)
     dist.init_process_group("gloo", rank=rank, world_size=n)
@@ -42,6 +43,7 @@ def _worker(rank, n, port, scheme, rate, recon, q):
         plan = kp.perf_plan("hotspot", W, h, 1, scheme, rate, recon)
         kp.perf_plan_set(plan, "global_h", H)
         kp.perf_plan_set(plan, "band_y0", y0)
+        kp.perf_plan_set(plan, "tblock", tb)
         hb = kp.perf_plan_get(plan, "halo_rows")
         kp.perf_destroy(plan)
         T0, P = synth.hotspot(synth.SEED_C4, W, H)
@@ -49,9 +51,9 @@ def _worker(rank, n, port, scheme, rate, recon, q):
         lo, hi = max(0, y0 - hb), min(H, y1 + hb)
         T = np.ascontiguousarray(T0[lo:hi].astype(np.float64))
         Pw = np.ascontiguousarray(P[lo:hi])
-        prm = oracle.params("hotspot", W, H, 1, scheme, rate, recon, 8)
+        prm = oracle.params("hotspot", W, H, 1, scheme, rate, recon, 8, tblock=tb)
         top = y0 - lo  # rows of top halo present
-        for _ in range(ITERS):
+        for i in range(0, ITERS, tb):
             reqs = []
             if rank > 0:  # my first hb rows up, its last hb rows into my top halo
                 reqs.append(dist.isend(torch.from_numpy(T[top:top + hb].copy()), rank - 1))
@@ -67,7 +69,7 @@ def _worker(rank, n, port, scheme, rate, recon, q):
                 T[:top] = buf_top.numpy()[hb - top:]
             if rank < n - 1:
                 T[top + h:] = buf_bot.numpy()[:hi - y1]
-            oracle.hotspot_window(prm, T, Pw, 0, lo, 1)
+            oracle.hotspot_window(prm, T, Pw, 0, lo, min(tb, ITERS - i))
         hmax = max(cuts[r + 1] - cuts[r] for r in range(n))  # gloo gathers equal shapes
         mine = torch.zeros((hmax, W), dtype=torch.float64)
         mine[:h] = torch.from_numpy(np.ascontiguousarray(T[top:top + h]))
@@ -82,14 +84,15 @@ def _worker(rank, n, port, scheme, rate, recon, q):
 
 
 @pytest.mark.parametrize("n", [2, 3])
-@pytest.mark.parametrize("scheme,rate,recon", [("none", (0, 1), "nn"), ("row", (1, 2), "li"),
-                                               ("row", (3, 4), "nn"), ("checker", (1, 4), "li"),
-                                               ("col", (1, 2), "li")])
-def test_banded_hotspot_equals_whole_grid(n, scheme, rate, recon):
+@pytest.mark.parametrize("scheme,rate,recon,tb", [("none", (0, 1), "nn", 1), ("row", (1, 2), "li", 1),
+                                                  ("row", (3, 4), "nn", 1), ("checker", (1, 4), "li", 1),
+                                                  ("col", (1, 2), "li", 1), ("row", (1, 2), "li", 3),
+                                                  ("none", (0, 1), "nn", 4)])
+def test_banded_hotspot_equals_whole_grid(n, scheme, rate, recon, tb):
     ctx = mp.get_context("spawn")
     q = ctx.Queue()
     port = _free_port()
-    procs = [ctx.Process(target=_worker, args=(r, n, port, scheme, rate, recon, q)) for r in range(n)]
+    procs = [ctx.Process(target=_worker, args=(r, n, port, scheme, rate, recon, q, tb)) for r in range(n)]
     for p in procs:
         p.start()
     got = q.get(timeout=120)
@@ -97,7 +100,7 @@ def test_banded_hotspot_equals_whole_grid(n, scheme, rate, recon):
         p.join(timeout=60)
         assert p.exitcode == 0
     T0, P = synth.hotspot(synth.SEED_C4, W, H)
-    want = oracle.hotspot(oracle.params("hotspot", W, H, 1, scheme, rate, recon, 8), T0, P, ITERS)
+    want = oracle.hotspot(oracle.params("hotspot", W, H, 1, scheme, rate, recon, 8, tblock=tb), T0, P, ITERS)
     assert np.array_equal(got, want)
 
 
@@ -110,4 +113,6 @@ def test_band_cuts_and_halo():
                                ("checker", (1, 8), 9), ("col", (1, 2), 1)]:
         h = kp.perf_plan("hotspot", 64, 64, 1, scheme, rate, "li")
         assert kp.perf_plan_get(h, "halo_rows") == want
+        kp.perf_plan_set(h, "tblock", 4)  # a launch of 4 steps reads 4 rows further
+        assert kp.perf_plan_get(h, "halo_rows") == want + 3
         kp.perf_destroy(h)
