@@ -300,6 +300,9 @@ def main():
     ap.add_argument("--no-variants", action="store_true")
     ap.add_argument("--no-cpu", action="store_true")
     ap.add_argument("--batch", type=int, default=0)
+    ap.add_argument("--halo", default="nccl", choices=["nccl", "p2p"],
+                    help="C4 with N > 1: halo exchange by NCCL send/recv or (NEXT-4) peer stores fused "
+                         "into the step kernels over NVLink (CUDA IPC + epoch flags)")
     ap.add_argument("--tblock", type=int, default=1,
                     help="C4 only: Hotspot steps per launch (temporal blocking, DESIGN.md R19); 1 = per-step")
     args = ap.parse_args()
@@ -507,7 +510,15 @@ def bench_hotspot(args, cfg, ws, rank, local, stream, peak, peak_src):
         keys.update(global_h=Hg, band_y0=y0)
     plan = kp.Plan("hotspot", W, h, 1, cfg["scheme"], cfg["rate"], cfg["recon"], **keys)
     exact = kp.Plan("hotspot", W, h, 1, "none", (0, 1), "nn", **keys)
-    if ws > 1:
+    if ws > 1 and args.halo == "p2p":  # NEXT-4: peer stores + flags, handles swapped once
+        import torch.distributed as dist
+        for pl in (plan, exact):
+            blobs = [None] * ws
+            dist.all_gather_object(blobs, kp.perf_p2p_export(pl.handle))
+            kp.perf_p2p_attach(pl.handle, blobs[rank - 1] if rank > 0 else None,
+                               blobs[rank + 1] if rank < ws - 1 else None)
+        barrier(ws)
+    elif ws > 1:
         import torch.distributed as dist
         uid = kp.perf_comm_unique_id() if rank == 0 else bytes(128)
         t = torch.tensor(list(uid), dtype=torch.uint8, device="cuda" if dist.get_backend() == "nccl" else "cpu")
@@ -564,12 +575,14 @@ def bench_hotspot(args, cfg, ws, rank, local, stream, peak, peak_src):
             "config": {"workload": cfg["workload"] + (f", temporal blocking {args.tblock} steps/launch"
                                                       if args.tblock > 1 else ""),
                        "bands": ws, "tblock": args.tblock,
-                       "halo": ("NCCL send/recv per launch" if ws > 1 else "none")},
+                       "halo": (("peer stores fused into the step kernel + epoch flags (NEXT-4)"
+                                 if args.halo == "p2p" else "NCCL send/recv per launch") if ws > 1 else "none")},
             "speedup_vs_exact": ms_ex / ms, "error": {"metric": "mre", "value": mre, "count": cnt},
             "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
                          "frac": achieved / peak, "traffic": None, "peak_source": peak_src,
                          "peak_mix": pmix, "frac_mix": achieved / pmix if pmix else None},
-            "clocks": clk.summary(), "gpu_launches": args.steps * (-(-iters // args.tblock)), "temporal_blocking": tblock}
+            "clocks": clk.summary(), "gpu_launches": args.steps * (-(-iters // args.tblock)) * (3 if ws > 1 and args.halo == "p2p" else 1),
+            "temporal_blocking": tblock}
 
 
 if __name__ == "__main__":

@@ -103,11 +103,16 @@ enum {
   PERF_KEY_TILE1_W = 12,       /* STENCIL1 tile width: power of two, 16..256 (fp32) / 16..512 (u8); default 16 */
   PERF_KEY_TILE1_H = 13,       /* STENCIL1 tile height, 1..1024; default 16 */
   PERF_KEY_PRODUCER = 14,      /* 0 auto = 1 dedicated producer warp; 2 bulk rows issued by consumer warp 0 */
-  PERF_KEY_TBLOCK = 15         /* Hotspot temporal blocking: steps per launch, 1..8 (default 1).  CHANGES
+  PERF_KEY_TBLOCK = 15,        /* Hotspot temporal blocking: steps per launch, 1..8 (default 1).  CHANGES
                                   RESULTS: T is loaded (perforated, rebuilt) once per launch and the other
                                   steps of the launch read on-chip T (R19).
-                                  NONE / ROW schemes; single-band plans */
+                                  NONE / ROW schemes; banded plans exchange TBLOCK + den halo rows per launch */
+  PERF_KEY_P2P = 16            /* perf_run_hotspot_bands_local only: 1 = halos by direct peer stores fused into
+                                  the step kernels + epoch flags (the NEXT-4 path), 0 = device copies */
 };
+
+/* size of a perf_p2p_export handle */
+#define PERF_P2P_HANDLE_BYTES 128
 
 /* Create a plan.  Validates: W, H >= 1; radius allowed for the app (Gaussian,
  * Sobel {1,2}; Median, Hotspot {1}; Gauss-Sobel {2}; Inversion {0});
@@ -157,6 +162,23 @@ perf_status perf_error(perf_plan_t plan, const void* exact, const void* approx, 
 perf_status perf_comm_init(perf_plan_t plan, const void* nccl_unique_id, int rank, int nranks);
 /* Fill a 128-byte buffer with a fresh ncclUniqueId (rank 0 calls this). */
 perf_status perf_comm_unique_id(void* out_128_bytes);
+
+/* NEXT-4: peer-memory halo exchange over NVLink / NVSwitch,
+ * replacing NCCL for the banded Hotspot.  perf_p2p_export allocates this
+ * band's buffers (band geometry: W, H, GLOBAL_H, BAND_Y0, scheme, TBLOCK must
+ * be final) and writes PERF_P2P_HANDLE_BYTES describing them (a CUDA IPC
+ * handle + geometry) for the neighbouring ranks.  perf_p2p_attach opens the
+ * upper (rank - 1) and lower (rank + 1) bands' handles (NULL at the grid
+ * edges) -- collective in the sense that every rank must attach before any
+ * rank runs.  Afterwards perf_run_hotspot stores each launch's first / last
+ * halo rows directly into the neighbours' buffers from inside the step
+ * kernel and orders launches with epoch flags (fence.sc.sys + st.release.sys
+ * / ld.acquire.sys polling); no NCCL call, no copy.  Every rank must run the
+ * same number of perf_run_hotspot calls with the same ITERS / TBLOCK.  The
+ * neighbours' processes must outlive the runs.  Errors: INVALID_ARG on a
+ * handle of another grid or a non-adjacent band, CUDA on IPC failures. */
+perf_status perf_p2p_export(perf_plan_t plan, void* handle_out);
+perf_status perf_p2p_attach(perf_plan_t plan, const void* up_handle, const void* down_handle);
 
 perf_status perf_destroy(perf_plan_t plan);
 const char* perf_last_error(void);

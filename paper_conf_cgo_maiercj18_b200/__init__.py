@@ -23,14 +23,14 @@ RECON = {"nn": 0, "li": 1, "linear": 1}
 METRIC = {"mre": 0, "me": 1, "mae": 2}
 KEY = {"batch": 1, "iters": 2, "granule_bytes": 3, "global_h": 4, "band_y0": 5, "tile_w": 6, "tile_h": 7,
        "metric": 8, "loader": 9, "ring": 10, "halo_rows": 11, "tile1_w": 12, "tile1_h": 13, "producer": 14,
-       "tblock": 15}
+       "tblock": 15, "p2p": 16}
 STATUS = {0: "PERF_OK", 1: "PERF_ERR_INVALID_ARG", 2: "PERF_ERR_UNSUPPORTED", 3: "PERF_ERR_CUDA",
           4: "PERF_ERR_NCCL", 5: "PERF_ERR_OOM"}
 
 # exported symbols of include/kperf.h (tests check the library exports all of them)
 SYMBOLS = ("perf_plan", "perf_plan_set", "perf_plan_get", "perf_run", "perf_run_host", "perf_run_hotspot",
            "perf_run_hotspot_bands_local", "perf_error", "perf_comm_init", "perf_comm_unique_id",
-           "perf_destroy", "perf_last_error", "perf_version")
+           "perf_p2p_export", "perf_p2p_attach", "perf_destroy", "perf_last_error", "perf_version")
 
 
 class PerfRate(ctypes.Structure):
@@ -65,6 +65,8 @@ def lib():
             "perf_error": [vp, vp, vp, vp, ctypes.POINTER(ctypes.c_double), ctypes.POINTER(ll)],
             "perf_comm_init": [vp, vp, i, i],
             "perf_comm_unique_id": [vp],
+            "perf_p2p_export": [vp, vp],
+            "perf_p2p_attach": [vp, vp, vp],
             "perf_destroy": [vp],
         }
         for name, args in sig.items():
@@ -164,6 +166,18 @@ def perf_comm_unique_id() -> bytes:
 def perf_comm_init(plan: int, unique_id: bytes, rank: int, nranks: int) -> None:
     buf = ctypes.create_string_buffer(bytes(unique_id), 128)
     _check(lib().perf_comm_init(plan, buf, rank, nranks))
+
+
+def perf_p2p_export(plan: int) -> bytes:
+    buf = ctypes.create_string_buffer(128)
+    _check(lib().perf_p2p_export(plan, buf))
+    return buf.raw
+
+
+def perf_p2p_attach(plan: int, up, down) -> None:
+    ub = ctypes.create_string_buffer(bytes(up), 128) if up is not None else None
+    db = ctypes.create_string_buffer(bytes(down), 128) if down is not None else None
+    _check(lib().perf_p2p_attach(plan, ub, db))
 
 
 def perf_destroy(plan: int) -> None:

@@ -52,6 +52,13 @@ struct KParams {
   int nrec;                  // recipe-table entries per consumer warp (>= n_recipes of a segment)
   int inline_prod;           // bulk loader issued by consumer warp 0 (no dedicated producer warp)
   float sdc, rx1, ry1, rz1, amb;  // Hotspot (Rodinia) coefficients
+  // NEXT-4 peer-memory halo exchange (banded Hotspot): output rows
+  // [y_begin, y_begin + halo_rows) are also stored into the upper neighbour's
+  // buffer pu (its row 0 = global row pu_row0), rows [y_end - halo_rows, y_end)
+  // into the lower neighbour's pd -- direct NVLink stores fused into the step
+  float* pu;
+  float* pd;
+  int pu_row0, pd_row0, halo_rows;
 };
 
 // compile-time loop: f(IC<0>{}), f(IC<1>{}), ... f(IC<N-1>{})

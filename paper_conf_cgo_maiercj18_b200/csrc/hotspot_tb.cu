@@ -230,15 +230,20 @@ __global__ void __launch_bounds__(32 * TB_WARPS, 3) hotspot_tb_kernel(const __gr
     const int gy = gy0 + q.apron + e;
     if (gy >= q.y_end) break;
     if (!mine) continue;
-    float* orow = q.out + (long long)(gy - q.out_row0) * q.W;
     const float4 v = ld4(fin + (q.apron + e) * TB_EW + 4 * lane);
-    if (q.vec && gx + 3 < q.W) {
-      st4(orow + gx, v);
-    } else {
+    auto put = [&](float* orow) {
+      if (q.vec && gx + 3 < q.W) {
+        st4(orow + gx, v);
+      } else {
 #pragma unroll
-      for (int k = 0; k < 4; ++k)
-        if (gx + k < q.W) orow[gx + k] = el(v, k);
-    }
+        for (int k = 0; k < 4; ++k)
+          if (gx + k < q.W) orow[gx + k] = el(v, k);
+      }
+    };
+    put(q.out + (long long)(gy - q.out_row0) * q.W);
+    // banded: boundary rows also go straight into the neighbours' buffers (NEXT-4)
+    if (q.pu && gy < q.y_begin + q.halo_rows) put(q.pu + (long long)(gy - q.pu_row0) * q.W);
+    if (q.pd && gy >= q.y_end - q.halo_rows) put(q.pd + (long long)(gy - q.pd_row0) * q.W);
   }
 }
 

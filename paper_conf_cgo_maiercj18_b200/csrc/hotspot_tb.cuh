@@ -18,6 +18,9 @@ struct TBParams {
   int vec;                                // 16-B loads allowed (W % 4 == 0, aligned buffers)
   float sdc, cx, cy, c0, pamb;             // sdc = step/Cap; cx = sdc/Rx, cy = sdc/Ry,
                                           // c0 = 1 - 2cx - 2cy - sdc/Rz, pamb = sdc amb / Rz (host, fp64 -> fp32)
+  float* pu;                              // NEXT-4 peer halo stores (see KParams in engine.cuh)
+  float* pd;
+  int pu_row0, pd_row0, halo_rows;
 };
 
 // S = q.steps (1..8) steps on output rows [y_begin, y_end); fills the tile geometry

@@ -151,22 +151,33 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
     }
   }
   // compute: the unchanged stencil on the rebuilt row (a3) and the store
+  int oy = ys;  // global row of the next output row
+  auto store = [&](T* dst, const Frag<T, V>& o) {
+    if (FAST && p.vec_io) {
+#pragma unroll
+      for (int q = 0; q < (int)(V * sizeof(T)) / 16; ++q) {
+        const uint4 u = reinterpret_cast<const uint4*>(&o)[q];
+        st_global_v4(dst + q * CV, u.x, u.y, u.z, u.w);
+      }
+    } else {
+#pragma unroll
+      for (int i = 0; i < V; ++i)
+        if (FAST || xc + i < p.W) dst[i] = o.get(i);
+    }
+  };
   auto compute = [&](auto uc, const Rows& r, int vy) {
     constexpr int U = decltype(uc)::value;
     const Frag<T, V> o = app.template row<U>(r.c, r.e, r.c2, lane, hf, vy, xc, p);
     if (r.emit) {  // kernel execution result -> output buffer (output rows in order)
-      if (FAST && p.vec_io) {
-#pragma unroll
-        for (int q = 0; q < (int)(V * sizeof(T)) / 16; ++q) {
-          const uint4 u = reinterpret_cast<const uint4*>(&o)[q];
-          st_global_v4(optr + q * CV, u.x, u.y, u.z, u.w);
-        }
-      } else {
-#pragma unroll
-        for (int i = 0; i < V; ++i)
-          if (FAST || xc + i < p.W) optr[i] = o.get(i);
+      store(optr, o);
+      if constexpr (App::NIN > 1) {  // banded Hotspot: boundary rows also go straight to the neighbours
+        if (p.pu && oy < p.y_begin + p.halo_rows)
+          store(reinterpret_cast<T*>(p.pu) + (long long)(oy - p.pu_row0) * p.W + xc, o);
+        if (p.pd && oy >= p.y_end - p.halo_rows)
+          store(reinterpret_cast<T*>(p.pd) + (long long)(oy - p.pd_row0) * p.W + xc, o);
       }
       optr += p.W;
+      ++oy;
     }
   };
 

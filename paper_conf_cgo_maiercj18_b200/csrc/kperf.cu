@@ -13,6 +13,7 @@
 
 #include "../../include/kperf.h"
 #include "hotspot_tb.cuh"
+#include "p2p.cuh"
 #include "kernel.cuh"
 
 namespace kp {
@@ -42,14 +43,33 @@ struct Band {  // banded Hotspot state
   int hb = 0;                 // halo rows each side
   float* buf[2] = {nullptr, nullptr};
   float* pbuf = nullptr;      // power with halo
+  unsigned* flags = nullptr;  // NEXT-4 epoch flags: [0] written by the upper band, [1] by the lower band
+  void* base = nullptr;       // one allocation: buf0 | buf1 | pbuf | flags (one CUDA IPC handle)
   size_t rows = 0;            // allocated rows (h + 2 hb)
+  // NEXT-4 peer links (perf_p2p_attach or bands_local with P2P)
+  bool p2p = false;
+  float* peer_buf[2][2] = {{nullptr, nullptr}, {nullptr, nullptr}};  // [0 upper / 1 lower band][parity]
+  float* peer_pbuf[2] = {nullptr, nullptr};
+  unsigned* peer_flag[2] = {nullptr, nullptr};  // my slot in the upper band (its flags[1]) / lower (its flags[0])
+  int peer_row0[2] = {0, 0};                    // global row of the neighbours' buffer row 0
+  void* peer_ipc[2] = {nullptr, nullptr};       // IPC mappings to close
+  unsigned epoch = 0;
 };
+
+// byte layout of a band allocation of `rows` x W floats per array
+struct BandLayout {
+  size_t arr, total;
+};
+static BandLayout band_layout(size_t rows, size_t W) {
+  const size_t arr = (rows * W * sizeof(float) + 255) & ~(size_t)255;
+  return {arr, 3 * arr + 256};
+}
 
 struct perf_plan_s {
   int app, W, H, radius, scheme, recon;
   perf_rate rate;
   long long batch = 1, iters = 1, granule_bytes = 128, global_h = -1, band_y0 = 0, tile_w = kp::kNCW, tile_h = 0,
-            metric = 0, loader = 0, ring = 0, tile1_w = 16, tile1_h = 16, producer = 0, tblock = 1;
+            metric = 0, loader = 0, ring = 0, tile1_w = 16, tile1_h = 16, producer = 0, tblock = 1, p2p = 0;
   double* d_err = nullptr;
   float* d_tmp = nullptr;
   size_t tmp_elems = 0;
@@ -347,6 +367,10 @@ perf_status perf_plan_set(perf_plan_t p, int key, long long v) {
       if (v < 1 || v > 8) return fail(PERF_ERR_INVALID_ARG, "TBLOCK must be in [1, 8]");
       p->tblock = v;
       return PERF_OK;
+    case PERF_KEY_P2P:
+      if (v < 0 || v > 1) return fail(PERF_ERR_INVALID_ARG, "P2P must be 0 or 1");
+      p->p2p = v;
+      return PERF_OK;
   }
   return fail(PERF_ERR_INVALID_ARG, "unknown key");
 }
@@ -369,6 +393,7 @@ perf_status perf_plan_get(perf_plan_t p, int key, long long* v) {
     case PERF_KEY_TILE1_H: *v = p->tile1_h; return PERF_OK;
     case PERF_KEY_PRODUCER: *v = p->producer; return PERF_OK;
     case PERF_KEY_TBLOCK: *v = p->tblock; return PERF_OK;
+    case PERF_KEY_P2P: *v = p->p2p; return PERF_OK;
   }
   return fail(PERF_ERR_INVALID_ARG, "unknown key");
 }
@@ -410,29 +435,46 @@ perf_status perf_run_host(perf_plan_t p, const void* host_in, void* host_out, vo
 }
 
 // ---------------------------------------------------------------- Hotspot ----
+static void band_free(perf_plan_s* p) {
+  for (void*& m : p->band.peer_ipc)
+    if (m) { cudaIpcCloseMemHandle(m); m = nullptr; }
+  if (p->band.base) cudaFree(p->band.base);
+  Band fresh;
+  p->band = fresh;
+}
+
 static perf_status band_alloc(perf_plan_s* p) {
   const int hb = band_halo(p);
   const size_t rows = (size_t)p->H + 2 * hb;
-  if (p->band.rows == rows && p->band.hb == hb) return PERF_OK;
-  for (float*& b : p->band.buf) if (b) { cudaFree(b); b = nullptr; }
-  if (p->band.pbuf) { cudaFree(p->band.pbuf); p->band.pbuf = nullptr; }
-  const size_t bytes = rows * p->W * sizeof(float);
-  if (cudaMalloc(&p->band.buf[0], bytes) != cudaSuccess || cudaMalloc(&p->band.buf[1], bytes) != cudaSuccess ||
-      cudaMalloc(&p->band.pbuf, bytes) != cudaSuccess)
-    return fail(PERF_ERR_OOM, "band allocation failed");
-  cudaMemset(p->band.buf[0], 0, bytes);
-  cudaMemset(p->band.buf[1], 0, bytes);
-  cudaMemset(p->band.pbuf, 0, bytes);
+  if (p->band.base && p->band.rows == rows && p->band.hb == hb) return PERF_OK;
+  if (p->band.p2p) return fail(PERF_ERR_INVALID_ARG, "band geometry changed after perf_p2p_attach");
+  band_free(p);
+  const BandLayout L = band_layout(rows, p->W);
+  void* base = nullptr;
+  if (cudaMalloc(&base, L.total) != cudaSuccess) return fail(PERF_ERR_OOM, "band allocation failed");
+  cudaMemset(base, 0, L.total);
+  char* b = static_cast<char*>(base);
+  p->band.base = base;
+  p->band.buf[0] = reinterpret_cast<float*>(b);
+  p->band.buf[1] = reinterpret_cast<float*>(b + L.arr);
+  p->band.pbuf = reinterpret_cast<float*>(b + 2 * L.arr);
+  p->band.flags = reinterpret_cast<unsigned*>(b + 3 * L.arr);
   p->band.rows = rows;
   p->band.hb = hb;
   return PERF_OK;
 }
 
 // one step of a band: rows [y0, y0+h) of buffer `src` (with halos filled) -> `dst`
-static perf_status band_step(perf_plan_s* p, const float* src, float* dst, int steps, cudaStream_t s) {
+static perf_status band_step(perf_plan_s* p, const float* src, float* dst, int steps, cudaStream_t s,
+                             float* pu = nullptr, float* pd = nullptr) {
   const int Hg = (int)p->global_h, y0 = (int)p->band_y0, h = p->H, hb = p->band.hb;
   if (p->tblock > 1) {  // `steps` steps in one temporally blocked launch
     kp::TBParams q = tb_params(p, src, p->band.pbuf, dst);
+    q.pu = pu;
+    q.pd = pd;
+    q.pu_row0 = p->band.peer_row0[0];
+    q.pd_row0 = p->band.peer_row0[1];
+    q.halo_rows = hb;
     q.in_row0 = q.out_row0 = y0 - hb;
     q.avail0 = std::max(0, y0 - hb);
     q.avail1 = std::min(Hg, y0 + h + hb);
@@ -450,6 +492,11 @@ static perf_status band_step(perf_plan_s* p, const float* src, float* dst, int s
                                y0 - hb, y0, y0 + h, k, grid, smem);
   if (st != PERF_OK) return st;
   k.in_fstride = k.out_fstride = 0;
+  k.pu = pu;
+  k.pd = pd;
+  k.pu_row0 = p->band.peer_row0[0];
+  k.pd_row0 = p->band.peer_row0[1];
+  k.halo_rows = hb;
   cudaError_t e = dispatch(p, k, grid, smem, s);
   if (e != cudaSuccess) return cuda_fail(e, "hotspot band launch");
   return PERF_OK;
@@ -471,6 +518,31 @@ static perf_status band_exchange_nccl(perf_plan_s* p, float* buf, cudaStream_t s
   ncclResult_t r = ncclGroupEnd();
   if (r != ncclSuccess) return fail(PERF_ERR_NCCL, std::string("halo exchange: ") + ncclGetErrorString(r));
   return PERF_OK;
+}
+
+// NEXT-4: push my boundary rows of `mine` (buffer rows [hb, 2hb) and [h, h+hb))
+// into the neighbours' halos `up`, `dn` (same parity) -- initial T and P only;
+// every later halo travels inside the step kernel
+static perf_status p2p_push(perf_plan_s* p, const float* mine, float* up, float* dn, cudaStream_t s) {
+  const size_t W = p->W, hb = p->band.hb, h = p->H;
+  const long long y0 = p->band_y0;
+  if (up)
+    CK(cudaMemcpyAsync(up + (y0 - p->band.peer_row0[0]) * (long long)W, mine + hb * W, hb * W * sizeof(float),
+                       cudaMemcpyDeviceToDevice, s));
+  if (dn)
+    CK(cudaMemcpyAsync(dn + (y0 + (long long)h - (long long)hb - p->band.peer_row0[1]) * (long long)W, mine + h * W,
+                       hb * W * sizeof(float), cudaMemcpyDeviceToDevice, s));
+  return PERF_OK;
+}
+static perf_status p2p_signal(perf_plan_s* p, cudaStream_t s) {
+  cudaError_t e = kp::p2p_signal(p->band.peer_flag[0], p->band.peer_flag[1], p->band.epoch + 1, s);
+  return e == cudaSuccess ? PERF_OK : cuda_fail(e, "p2p signal");
+}
+static perf_status p2p_wait(perf_plan_s* p, cudaStream_t s) {
+  ++p->band.epoch;
+  cudaError_t e = kp::p2p_wait(p->band.flags, p->band.peer_flag[0] != nullptr, p->band.peer_flag[1] != nullptr,
+                               p->band.epoch, s);
+  return e == cudaSuccess ? PERF_OK : cuda_fail(e, "p2p wait");
 }
 
 perf_status perf_run_hotspot(perf_plan_t p, const float* temp_in, const float* power, float* temp_out, void* stream) {
@@ -532,8 +604,9 @@ perf_status perf_run_hotspot(perf_plan_t p, const float* temp_in, const float* p
     return PERF_OK;
   }
   // banded: this rank owns global rows [band_y0, band_y0 + H) of Hg
-  if (!p->comm && p->nranks == 1 && Hg != p->H)
-    return fail(PERF_ERR_INVALID_ARG, "banded Hotspot needs perf_comm_init (or perf_run_hotspot_bands_local)");
+  if (!p->comm && !p->band.p2p && p->nranks == 1 && Hg != p->H)
+    return fail(PERF_ERR_INVALID_ARG,
+                "banded Hotspot needs perf_comm_init or perf_p2p_attach (or perf_run_hotspot_bands_local)");
   perf_status st = band_alloc(p);
   if (st != PERF_OK) return st;
   const int hb = p->band.hb;
@@ -541,6 +614,23 @@ perf_status perf_run_hotspot(perf_plan_t p, const float* temp_in, const float* p
   const size_t W = p->W;
   CK(cudaMemcpyAsync(p->band.buf[0] + hb * W, temp_in, n * sizeof(float), cudaMemcpyDeviceToDevice, s));
   CK(cudaMemcpyAsync(p->band.pbuf + hb * W, power, n * sizeof(float), cudaMemcpyDeviceToDevice, s));
+  if (p->band.p2p) {  // NEXT-4: halos by direct peer stores fused into the step kernels, epoch flags
+    Band& B = p->band;
+    if ((st = p2p_push(p, B.buf[0], B.peer_buf[0][0], B.peer_buf[1][0], s)) != PERF_OK) return st;
+    if ((st = p2p_push(p, B.pbuf, B.peer_pbuf[0], B.peer_pbuf[1], s)) != PERF_OK) return st;
+    if ((st = p2p_signal(p, s)) != PERF_OK || (st = p2p_wait(p, s)) != PERF_OK) return st;
+    int cur = 0;
+    for (long long i = 0; i < p->iters; i += p->tblock) {
+      const int steps = (int)std::min(p->tblock, p->iters - i);
+      if ((st = band_step(p, B.buf[cur], B.buf[cur ^ 1], steps, s, B.peer_buf[0][cur ^ 1], B.peer_buf[1][cur ^ 1])) !=
+          PERF_OK)
+        return st;
+      if ((st = p2p_signal(p, s)) != PERF_OK || (st = p2p_wait(p, s)) != PERF_OK) return st;
+      cur ^= 1;
+    }
+    CK(cudaMemcpyAsync(temp_out, B.buf[cur] + hb * W, n * sizeof(float), cudaMemcpyDeviceToDevice, s));
+    return PERF_OK;
+  }
   if ((st = band_exchange_nccl(p, p->band.pbuf, s)) != PERF_OK) return st;
   int cur = 0;
   for (long long i = 0; i < p->iters; i += p->tblock) {  // one halo exchange + launch per TBLOCK steps
@@ -597,10 +687,68 @@ perf_status perf_run_hotspot_bands_local(perf_plan_t* plans, int nb, const float
     }
     return PERF_OK;
   };
-  perf_status st = exchange(0, true);
+  perf_status st;
+  const long long tb = plans[0]->tblock;
+  if (plans[0]->p2p) {  // NEXT-4 emulated on one device: direct peer stores + epoch flags, no copies
+    for (int b = 0; b < nb; ++b) {  // wire neighbours' band buffers as the peers
+      Band& B = plans[b]->band;
+      if (b > 0) {
+        Band& U = plans[b - 1]->band;
+        if (U.hb != B.hb) return fail(PERF_ERR_INVALID_ARG, "band plans must share the halo size");
+        B.peer_buf[0][0] = U.buf[0];
+        B.peer_buf[0][1] = U.buf[1];
+        B.peer_pbuf[0] = U.pbuf;
+        B.peer_flag[0] = U.flags + 1;
+        B.peer_row0[0] = (int)plans[b - 1]->band_y0 - U.hb;
+      }
+      if (b < nb - 1) {
+        Band& D = plans[b + 1]->band;
+        B.peer_buf[1][0] = D.buf[0];
+        B.peer_buf[1][1] = D.buf[1];
+        B.peer_pbuf[1] = D.pbuf;
+        B.peer_flag[1] = D.flags;
+        B.peer_row0[1] = (int)plans[b + 1]->band_y0 - D.hb;
+      }
+      B.p2p = true;
+    }
+    for (int b = 0; b < nb; ++b) {
+      Band& B = plans[b]->band;
+      if ((st = p2p_push(plans[b], B.buf[0], B.peer_buf[0][0], B.peer_buf[1][0], s)) != PERF_OK) return st;
+      if ((st = p2p_push(plans[b], B.pbuf, B.peer_pbuf[0], B.peer_pbuf[1], s)) != PERF_OK) return st;
+    }
+    // one stream: every band's launch, then every band's signal, then every wait
+    auto sync_all = [&]() -> perf_status {
+      perf_status r;
+      for (int b = 0; b < nb; ++b)
+        if ((r = p2p_signal(plans[b], s)) != PERF_OK) return r;
+      for (int b = 0; b < nb; ++b)
+        if ((r = p2p_wait(plans[b], s)) != PERF_OK) return r;
+      return PERF_OK;
+    };
+    if ((st = sync_all()) != PERF_OK) return st;
+    int cur = 0;
+    for (long long i = 0; i < iters; i += tb) {
+      const int steps = (int)std::min(tb, iters - i);
+      for (int b = 0; b < nb; ++b) {
+        Band& B = plans[b]->band;
+        if ((st = band_step(plans[b], B.buf[cur], B.buf[cur ^ 1], steps, s, B.peer_buf[0][cur ^ 1],
+                            B.peer_buf[1][cur ^ 1])) != PERF_OK)
+          return st;
+      }
+      if ((st = sync_all()) != PERF_OK) return st;
+      cur ^= 1;
+    }
+    for (int b = 0; b < nb; ++b) {
+      perf_plan_s* p = plans[b];
+      CK(cudaMemcpyAsync(temp_out + (size_t)p->band_y0 * W, p->band.buf[cur] + (size_t)p->band.hb * W,
+                         (size_t)p->H * W * sizeof(float), cudaMemcpyDeviceToDevice, s));
+      p->band.p2p = false;  // (local wiring is per call)
+    }
+    return PERF_OK;
+  }
+  st = exchange(0, true);
   if (st != PERF_OK) return st;
   int cur = 0;
-  const long long tb = plans[0]->tblock;
   for (long long i = 0; i < iters; i += tb) {
     if ((st = exchange(cur, false)) != PERF_OK) return st;
     const int steps = (int)std::min(tb, iters - i);
@@ -662,14 +810,73 @@ perf_status perf_comm_init(perf_plan_t p, const void* uid, int rank, int nranks)
   return PERF_OK;
 }
 
+// ------------------------------------------------------- NEXT-4 peer links ----
+namespace {
+struct P2PBlob {  // what perf_p2p_export writes (PERF_P2P_HANDLE_BYTES = 128)
+  uint32_t magic, W, H, hb;
+  int32_t band_y0, pad[3];
+  cudaIpcMemHandle_t handle;  // 64 bytes
+};
+static_assert(sizeof(P2PBlob) <= 128, "blob size");
+constexpr uint32_t kP2PMagic = 0x4B503250u;  // "P2PK"
+}  // namespace
+
+perf_status perf_p2p_export(perf_plan_t p, void* out) {
+  if (!p || !out) return fail(PERF_ERR_INVALID_ARG, "NULL argument");
+  if (p->app != PERF_APP_HOTSPOT) return fail(PERF_ERR_INVALID_ARG, "P2P halos are for banded Hotspot plans");
+  perf_status st = band_alloc(p);
+  if (st != PERF_OK) return st;
+  P2PBlob b;
+  std::memset(&b, 0, sizeof b);
+  b.magic = kP2PMagic;
+  b.W = (uint32_t)p->W;
+  b.H = (uint32_t)p->H;
+  b.hb = (uint32_t)p->band.hb;
+  b.band_y0 = (int32_t)p->band_y0;
+  CK(cudaIpcGetMemHandle(&b.handle, p->band.base));
+  std::memset(out, 0, PERF_P2P_HANDLE_BYTES);
+  std::memcpy(out, &b, sizeof b);
+  return PERF_OK;
+}
+
+perf_status perf_p2p_attach(perf_plan_t p, const void* up, const void* down) {
+  if (!p) return fail(PERF_ERR_INVALID_ARG, "NULL plan");
+  perf_status st = band_alloc(p);
+  if (st != PERF_OK) return st;
+  Band& B = p->band;
+  const void* blobs[2] = {up, down};
+  for (int k = 0; k < 2; ++k) {
+    if (!blobs[k]) continue;
+    P2PBlob b;
+    std::memcpy(&b, blobs[k], sizeof b);
+    if (b.magic != kP2PMagic || (int)b.W != p->W || (int)b.hb != B.hb)
+      return fail(PERF_ERR_INVALID_ARG, "peer handle: not a band of this grid (W / halo mismatch)");
+    const long long adj = k == 0 ? (long long)b.band_y0 + b.H : (long long)p->band_y0 + p->H;
+    if (adj != (k == 0 ? p->band_y0 : (long long)b.band_y0))
+      return fail(PERF_ERR_INVALID_ARG, "peer handle: band is not adjacent");
+    void* m = nullptr;
+    CK(cudaIpcOpenMemHandle(&m, b.handle, cudaIpcMemLazyEnablePeerAccess));
+    const BandLayout L = band_layout((size_t)b.H + 2 * b.hb, b.W);
+    char* base = static_cast<char*>(m);
+    B.peer_ipc[k] = m;
+    B.peer_buf[k][0] = reinterpret_cast<float*>(base);
+    B.peer_buf[k][1] = reinterpret_cast<float*>(base + L.arr);
+    B.peer_pbuf[k] = reinterpret_cast<float*>(base + 2 * L.arr);
+    // my slot in the neighbour's flags: the upper band reads "from lower" (1), the lower "from upper" (0)
+    B.peer_flag[k] = reinterpret_cast<unsigned*>(base + 3 * L.arr) + (k == 0 ? 1 : 0);
+    B.peer_row0[k] = b.band_y0 - (int)b.hb;
+  }
+  B.p2p = true;
+  return PERF_OK;
+}
+
 perf_status perf_destroy(perf_plan_t p) {
   if (!p) return PERF_OK;
   if (p->d_err) cudaFree(p->d_err);
   if (p->d_tmp) cudaFree(p->d_tmp);
   if (p->d_stage_in) cudaFree(p->d_stage_in);
   if (p->d_stage_out) cudaFree(p->d_stage_out);
-  for (float* b : p->band.buf) if (b) cudaFree(b);
-  if (p->band.pbuf) cudaFree(p->band.pbuf);
+  band_free(p);
   if (p->comm) ncclCommDestroy(p->comm);
   delete p;
   return PERF_OK;

@@ -286,6 +286,85 @@ def test_hotspot_bands_equal_whole_grid(scheme, rate, recon, nb, tb):
         q.close()
 
 
+@pytest.mark.parametrize("scheme,rate,recon,tb", [("none", (0, 1), "nn", 1), ("row", (1, 2), "li", 1),
+                                                  ("row", (3, 4), "nn", 1), ("checker", (1, 2), "li", 1),
+                                                  ("col", (1, 4), "nn", 1), ("row", (1, 2), "li", 4),
+                                                  ("none", (0, 1), "nn", 8)])
+@pytest.mark.parametrize("nb", [2, 3])
+def test_hotspot_p2p_bands_equal_whole_grid(scheme, rate, recon, tb, nb):
+    """NEXT-4 on one device: halo rows stored by the step kernels straight into
+    the neighbours' band buffers + epoch flags == one grid, bit for bit."""
+    W, H, iters = 640, 200, 9
+    T, P = synth.hotspot(17, W, H)
+    Td, Pd = torch.from_numpy(T).cuda(), torch.from_numpy(P).cuda()
+    whole = torch.empty_like(Td)
+    with kp.Plan("hotspot", W, H, 1, scheme, rate, recon, iters=iters, tblock=tb) as p:
+        p.hotspot(Td, Pd, whole)
+    cuts = np.linspace(0, H, nb + 1).astype(int)
+    cuts[1:-1] -= 5  # uneven bands
+    plans = [kp.Plan("hotspot", W, int(cuts[b + 1] - cuts[b]), 1, scheme, rate, recon, iters=iters, global_h=H,
+                     band_y0=int(cuts[b]), tblock=tb, p2p=1) for b in range(nb)]
+    banded = torch.full_like(Td, float("nan"))
+    for _ in range(2):  # twice: the epoch counters carry across calls
+        kp.perf_run_hotspot_bands_local([q.handle for q in plans], Td, Pd, banded)
+        torch.cuda.synchronize()
+        assert torch.equal(banded, whole)
+    for q in plans:
+        q.close()
+
+
+def _p2p_worker(rank, n, W, H, iters, tb, scheme, rate, recon, blobs, barrier, out_q):
+    import torch as t
+    import paper_conf_cgo_maiercj18_b200 as kp2
+    import synth as sy
+    t.cuda.set_device(0)
+    cuts = kp2.band_cuts(H, n)
+    y0, h = cuts[rank], cuts[rank + 1] - cuts[rank]
+    T, P = sy.hotspot(23, W, H)
+    Td = t.from_numpy(np.ascontiguousarray(T[y0:y0 + h])).cuda()
+    Pd = t.from_numpy(np.ascontiguousarray(P[y0:y0 + h])).cuda()
+    out = t.empty_like(Td)
+    with kp2.Plan("hotspot", W, h, 1, scheme, rate, recon, iters=iters, global_h=H, band_y0=y0, tblock=tb) as p:
+        blobs[rank] = kp2.perf_p2p_export(p.handle)
+        barrier.wait(timeout=120)
+        kp2.perf_p2p_attach(p.handle, blobs[rank - 1] if rank > 0 else None, blobs[rank + 1] if rank < n - 1 else None)
+        barrier.wait(timeout=120)  # every rank attached before any rank runs
+        p.hotspot(Td, Pd, out)
+        t.cuda.synchronize()
+        out_q.put((rank, out.cpu().numpy()))
+        barrier.wait(timeout=300)  # the neighbours' buffers stay mapped until everyone is done
+
+
+@pytest.mark.parametrize("scheme,rate,recon,tb", [("row", (1, 2), "li", 1), ("row", (1, 2), "li", 4)])
+def test_hotspot_p2p_ipc_two_processes(scheme, rate, recon, tb):
+    """NEXT-4 through real CUDA IPC: two processes (two contexts on this one
+    GPU) run adjacent bands with perf_p2p_export / perf_p2p_attach; the halo
+    stores and flags cross the process boundary.  == one grid, bit for bit."""
+    import torch.multiprocessing as mp
+    W, H, iters, n = 520, 96, 6, 2
+    T, P = synth.hotspot(23, W, H)
+    Td, Pd = torch.from_numpy(T).cuda(), torch.from_numpy(P).cuda()
+    whole = torch.empty_like(Td)
+    with kp.Plan("hotspot", W, H, 1, scheme, rate, recon, iters=iters, tblock=tb) as p:
+        p.hotspot(Td, Pd, whole)
+    torch.cuda.synchronize()
+    ctx = mp.get_context("spawn")
+    mgr = ctx.Manager()
+    blobs = mgr.dict()
+    barrier = mgr.Barrier(n)
+    out_q = ctx.Queue()
+    procs = [ctx.Process(target=_p2p_worker, args=(r, n, W, H, iters, tb, scheme, rate, recon, blobs, barrier, out_q))
+             for r in range(n)]
+    for pr in procs:
+        pr.start()
+    parts = dict(out_q.get(timeout=300) for _ in range(n))
+    for pr in procs:
+        pr.join(timeout=120)
+        assert pr.exitcode == 0
+    got = np.concatenate([parts[r] for r in range(n)])
+    assert np.array_equal(got, whole.cpu().numpy())
+
+
 # ---------------------------------------------------------------------------
 # Hotspot temporal blocking (SURVEY NEXT-3, DESIGN.md R19): TBLOCK steps per
 # launch, T perforated at the first step of each launch -- oracle `tblock`
