@@ -97,6 +97,42 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
   const int nv = n_recipes<SCHEME>(p, ys, ye, VR);  // virtual input rows of this segment
   int ready = g0 - 1, released = g0;  // this warp's ring counters (global load indices)
 
+  // column scheme, u8, NN: which bytes of a lane's chunk take the left /
+  // right neighbour granule's edge sample is row-independent -- byte masks
+  // hoisted out of the row loop; the per-row rebuild is then branch-free:
+  // word = (loaded & km) | (a x 0x01010101 & ma) | (b x 0x01010101 & mb)
+  struct NNu8 {
+    int ca, cb;       // ring columns of the edge samples a (left) and b (right)
+    uint32_t km;      // ~0: the chunk is loaded
+    uint32_t ma[4], mb[4];
+  };
+  auto nn_u8 = [&](const ChunkInfo& ci, int fx, int col, int nbytes) {
+    NNu8 z;
+    const bool kept = ci.col_kept;
+    const bool hb = ci.xb >= 0;
+    z.km = kept ? ~0u : 0u;
+    z.ca = kept ? col : ci.xa - base;
+    z.cb = (kept || !hb) ? z.ca : ci.xb - base;
+    const int lim = ci.xa + ci.xb - 2 * fx;  // byte i takes a iff 2 i <= lim (ties to the lower column)
+#pragma unroll
+    for (int k = 0; k < 4; ++k) {
+      uint32_t ma = 0, all = 0;
+#pragma unroll
+      for (int j = 0; j < 4; ++j) {
+        const int i = 4 * k + j;
+        if (i < nbytes) all |= 0xFFu << (8 * j);
+        if (i < nbytes && (!hb || 2 * i <= lim)) ma |= 0xFFu << (8 * j);
+      }
+      z.ma[k] = kept ? 0u : ma;
+      z.mb[k] = kept ? 0u : (all & ~ma);
+    }
+    return z;
+  };
+  NNu8 zc, ze;
+  if constexpr (SCHEME == S_COL && sizeof(T) == 1 && RECON == R_NN && FAST) {
+    zc = nn_u8(cc, xc, ccol, V);
+    ze = nn_u8(ce, ex, ecol, EW);
+  }
   struct Rows {  // one rebuilt input row as the lane sees it
     Frag<T, V> c, c2;
     Frag<T, EW> e;
@@ -120,7 +156,21 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
       ++ready;
       mbar_wait_u32(full_u32 + 8 * (ready & nmask), (ready >> p.nr_log2) & 1);
     }
-    if (FAST) {
+    if constexpr (FAST && SCHEME == S_COL && sizeof(T) == 1 && RECON == R_NN) {
+      const T* row = ring + rc_slot_a(rec.info) * slot_elems;
+      auto combine = [&](auto nc, const NNu8& z, int col) {
+        constexpr int N = decltype(nc)::value;
+        Frag<T, N> f = ldf<T, N>(row + col);
+        const uint32_t wa = 0x01010101u * (uint32_t)row[z.ca], wb = 0x01010101u * (uint32_t)row[z.cb];
+#pragma unroll
+        for (int k = 0; k < N / 4; ++k) f.w[k] = (f.w[k] & z.km) | (wa & z.ma[k]) | (wb & z.mb[k]);
+        return f;
+      };
+      r.c = combine(IC<V>{}, zc, ccol);
+      const Frag<T, EW> el = combine(IC<EW>{}, ze, ecol);
+      const Frag<T, EW> eb = Frag<T, EW>::splat(emode == 1 ? r.c.get(0) : r.c.get(V - 1));
+      r.e = emode == 0 ? el : eb;
+    } else if (FAST) {
       r.c = rebuild_frag<T, V, SCHEME, RECON>(p, m, rp, rec, cc, ring, slot_elems, ccol, xc, base);
       if (App::NIN > 1) r.c2 = rebuild_frag<T, V, SCHEME, RECON>(p, m, rp, rec, cc, ring2, slot_elems, ccol, xc, base);
       // edge fragment: loaded (inside the image) or the clamped border sample -- selects, no branch
