@@ -201,7 +201,9 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
     }
   }
   // compute: the unchanged stencil on the rebuilt row (a3) and the store
-  int oy = ys;  // global row of the next output row
+  // banded Hotspot: does this segment emit rows the neighbours need?  (CTA-uniform)
+  const bool peer_seg = App::NIN > 1 && p.halo_rows > 0 && (p.pu || p.pd) &&
+                        (ys < p.y_begin + p.halo_rows || ye > p.y_end - p.halo_rows);
   auto store = [&](T* dst, const Frag<T, V>& o) {
     if (FAST && p.vec_io) {
 #pragma unroll
@@ -221,13 +223,15 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
     if (r.emit) {  // kernel execution result -> output buffer (output rows in order)
       store(optr, o);
       if constexpr (App::NIN > 1) {  // banded Hotspot: boundary rows also go straight to the neighbours
-        if (p.pu && oy < p.y_begin + p.halo_rows)
-          store(reinterpret_cast<T*>(p.pu) + (long long)(oy - p.pu_row0) * p.W + xc, o);
-        if (p.pd && oy >= p.y_end - p.halo_rows)
-          store(reinterpret_cast<T*>(p.pd) + (long long)(oy - p.pd_row0) * p.W + xc, o);
+        if (peer_seg) {
+          const int oy = vy - VR;  // global output row (not Stencil1: emitted row = virtual row - VR)
+          if (p.pu && oy < p.y_begin + p.halo_rows)
+            store(reinterpret_cast<T*>(p.pu) + (long long)(oy - p.pu_row0) * p.W + xc, o);
+          if (p.pd && oy >= p.y_end - p.halo_rows)
+            store(reinterpret_cast<T*>(p.pd) + (long long)(oy - p.pd_row0) * p.W + xc, o);
+        }
       }
       optr += p.W;
-      ++oy;
     }
   };
 
@@ -373,7 +377,18 @@ cudaError_t launch_one(const KParams& p, unsigned grid, size_t smem, cudaStream_
   // of row segments so the CTA count fills whole waves of resident CTA slots
   // (occupancy API), discounted by the per-segment halo rows.
   KParams q = p;
-  if (p.seg_auto) {
+  // fp32 whole-row (TMA bulk) loaders, one input, radius <= 2: fixed 64-row
+  // segments -- several waves of short items balance better than the
+  // wave-filling choice below (C2: row 1/2 0.178 -> 0.170 ms, exact 0.193 ->
+  // 0.181 ms; tools/sweep_tile_h.py).  Cell loaders, u8, Hotspot and the
+  // fused pipeline measured best with the wave-filling choice.
+  const bool fixed64 = p.seg_auto && p.loader == L_BULK && App::VR <= 2 && App::NIN == 1 && sizeof(typename App::T) == 4 &&
+                       SCHEME != S_STENCIL1;
+  if (fixed64) {
+    q.seg_h = 64;
+    q.n_segs = (p.y_end - p.y_begin + 63) / 64;
+    grid = (unsigned)((long long)q.n_strips * q.n_segs * q.frames);
+  } else if (p.seg_auto) {
     static int per_sm = 0, sms = 0;
     static size_t per_sm_smem = 0;
     if (per_sm == 0 || per_sm_smem != smem) {
@@ -390,9 +405,10 @@ cudaError_t launch_one(const KParams& p, unsigned grid, size_t smem, cudaStream_
     const int rows = p.y_end - p.y_begin;
     const long long per_seg = (long long)p.n_strips * p.frames;
     double best = -1.0;
-    int best_n = (rows + p.seg_h - 1) / p.seg_h;
+    const int seg_cap = p.seg_h;
+    int best_n = (rows + seg_cap - 1) / seg_cap;
     const int th = SCHEME == S_STENCIL1 ? p.tile1_h : 1;  // Stencil1 segments hold whole tiles
-    for (int n = (rows + p.seg_h - 1) / p.seg_h; n <= (rows + 31) / 32 && n <= 4 * best_n + 64; ++n) {
+    for (int n = (rows + seg_cap - 1) / seg_cap; n <= (rows + 31) / 32 && n <= 4 * best_n + 64; ++n) {
       const int sh = ((rows + n - 1) / n + th - 1) / th * th;
       const int nn = (rows + sh - 1) / sh;
       const long long items = per_seg * nn;
