@@ -545,7 +545,9 @@ def bench_hotspot(args, cfg, ws, rank, local, stream, peak, peak_src):
     ms_ex = max_over_ranks(ws, time_kernel(lambda: exact.hotspot(T, P, out_ex, stream), stream, 2, 1))
     mre, cnt = plan.error(out_ex, out, stream)
     cells = W * Hg * iters
-    algo_b = bytes_per_px("hotspot", cfg["scheme"], cfg["rate"]) * W * h * iters
+    # per launch: kept T + P read and T' written once; a launch covers tblock
+    # steps under temporal blocking, one step otherwise
+    algo_b = bytes_per_px("hotspot", cfg["scheme"], cfg["rate"]) * W * h * iters / max(args.tblock, 1)
     achieved = algo_b / (ms * 1e-3) / 1e9
     # NEXT-3 temporal blocking (single band only): TBLOCK steps per launch, T
     # perforated once per launch (R19) -- reported next to the
