@@ -28,14 +28,17 @@ NVCC_FLAGS = ["-gencode", "arch=compute_100a,code=sm_100a", "-std=c++17", "-O3",
               "-Xcompiler", "-fPIC", "-Xptxas", "-v"]
 
 
-def build(force: bool = False, verbose: bool = False, defines=(), out=None) -> str:
-    srcs = sorted(glob.glob(os.path.join(CSRC, "*.cu")))
-    deps = srcs + glob.glob(os.path.join(CSRC, "*.cuh")) + [os.path.join(ROOT, "include", "kperf.h")]
+def build(force: bool = False, verbose: bool = False, defines=(), out=None, csrc=None) -> str:
+    csrc = csrc or CSRC  # (experiment builds: a snapshot of csrc/, see tools/ab.py)
+    srcs = sorted(glob.glob(os.path.join(csrc, "*.cu")))
+    deps = srcs + glob.glob(os.path.join(csrc, "*.cuh")) + [os.path.join(ROOT, "include", "kperf.h")]
     newest = max(os.path.getmtime(f) for f in deps)
     lib = out or LIB
     if not force and os.path.exists(lib) and os.path.getmtime(lib) >= newest:
         return lib
     objdir = OBJ if not defines else OBJ + "_" + "_".join(d.replace("=", "") for d in defines)
+    if out:
+        objdir = os.path.join(os.path.dirname(os.path.abspath(out)), "obj")
     os.makedirs(objdir, exist_ok=True)
     nccl = _nccl_dir()
     inc = ["-I", os.path.join(nccl, "include"), "-I", os.path.join(ROOT, "include")]
@@ -67,4 +70,6 @@ def build(force: bool = False, verbose: bool = False, defines=(), out=None) -> s
 if __name__ == "__main__":
     defs = [a[2:] for a in sys.argv[1:] if a.startswith("-D")]
     outs = [a[6:] for a in sys.argv[1:] if a.startswith("--out=")]
-    print(build(force="--force" in sys.argv, verbose="-v" in sys.argv, defines=defs, out=outs[0] if outs else None))
+    srcd = [a[7:] for a in sys.argv[1:] if a.startswith("--csrc=")]
+    print(build(force="--force" in sys.argv, verbose="-v" in sys.argv, defines=defs, out=outs[0] if outs else None,
+                csrc=srcd[0] if srcd else None))

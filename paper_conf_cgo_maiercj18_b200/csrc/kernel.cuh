@@ -42,7 +42,8 @@ __device__ __forceinline__ void mbar_arrive_u32(uint32_t addr) {
 template <class App, int SCHEME, int RECON, int NCW, bool FAST>
 __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int x0, int frame,
                                          int ys, int ye, int g0, uint32_t full_u32, uint32_t empty_u32,
-                                         const typename App::T* ring, int slot_elems, const Recipe* rtab) {
+                                         const typename App::T* ring, int slot_elems, const Recipe* rtab,
+                                         float4* ctab) {
   using T = typename App::T;
   constexpr int V = App::V, EW = App::EW, VR = App::VR, NWIN = App::NWIN;
   constexpr int CV = 16 / sizeof(T);  // elements of one 16-B mask-uniform chunk
@@ -133,6 +134,66 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
     zc = nn_u8(cc, xc, ccol, V);
     ze = nn_u8(ce, ex, ecol, EW);
   }
+  // column scheme, fp32: the rebuild of a lane's chunk is row independent
+  // except for the two edge samples a, b of the neighbouring loaded granules,
+  // so the per-lane facts are hoisted and the per-row work is branch free:
+  //   c = own samples (garbage unless kept), a = row[ca], b = row[cb]
+  //   LI: r_i = fmaf(a - b, w_i, b), w_i = (xb - x_i) / (xb - xa) from a
+  //       per-lane shared-memory table (same arithmetic as rebuild_frag)
+  //   NN: r_i = (2 i <= lim) ? a : b   (lanes wholly on one side: ca = cb)
+  //   out_i = kept ? c_i : r_i
+  // (the former divergent kept / skipped branch ran both sides per warp)
+  struct ColF {
+    int ca, cb, lim;
+    bool kept;
+  };
+  constexpr bool COLF = FAST && SCHEME == S_COL && sizeof(T) == 4;
+  auto colf_of = [&](const ChunkInfo& ci, int fx, int col, int n, float4* wt) {
+    ColF z;
+    z.kept = ci.col_kept;
+    const bool hb = ci.xb >= 0;
+    z.ca = z.kept ? col : ci.xa - base;
+    z.cb = (z.kept || !hb) ? z.ca : ci.xb - base;
+    z.lim = hb ? ci.xa + ci.xb - 2 * fx : 2 * n;  // sample i takes a iff 2 i <= lim
+    if (RECON == R_NN && !z.kept && z.lim >= 2 * (n - 1)) z.cb = z.ca;  // NN: all samples take a
+    else if (RECON == R_NN && !z.kept && z.lim < 0) z.ca = z.cb;        // NN: all take b
+    if (RECON == R_LI) {
+      float w[8] = {0.f, 0.f, 0.f, 0.f, 0.f, 0.f, 0.f, 0.f};
+      if (!z.kept && hb) {
+        const float inv = __frcp_rn((float)(ci.xb - ci.xa)), x0 = (float)(ci.xb - fx);
+#pragma unroll
+        for (int i = 0; i < 8; ++i)
+          if (i < n) w[i] = __fmul_rn(x0 - (float)i, inv);
+      }
+      wt[0] = make_float4(w[0], w[1], w[2], w[3]);
+      if (n > 4) wt[32] = make_float4(w[4], w[5], w[6], w[7]);
+    }
+    return z;
+  };
+  // checkerboard, fp32: per-lane slot choice instead of a divergent kept /
+  // skipped branch; every lane then loads one (NN) or two (LI) ring rows and
+  // LI is the row scheme's lerp b + (a - b) * wa (exact when a == b, i.e. for
+  // kept lanes and the NN fallback), wa = db / (da + db) from a per-warp table
+  // (LI only: for NN the old per-lane branch is just one load on either side and
+  // measured faster -- sobel3 checker 1/4 NN 230 -> 252 us with the slot select)
+  constexpr bool CHKF = FAST && SCHEME == S_CHECKER && sizeof(T) == 4 && RECON == R_LI;
+  if constexpr (CHKF) {
+    if (lane < m.den) {
+      const int t = lane;
+      reinterpret_cast<float*>(ctab)[t] =
+          m.phase_kept(t) ? 1.f : __fdiv_rn((float)m.dhi(t), (float)(m.dlo(t) + m.dhi(t)));
+    }
+    __syncwarp();
+  }
+  ColF fc, fe;
+  bool nn_mixed = false;  // some lane's chunk straddles the NN midpoint (G/2 not a multiple of V)
+  if constexpr (COLF) {
+    fc = colf_of(cc, xc, ccol, V, ctab + lane);
+    fe = colf_of(ce, ex, ecol, EW, ctab + 64 + lane);
+    const bool mixed = (!fc.kept && fc.ca != fc.cb) || (!fe.kept && fe.ca != fe.cb);
+    nn_mixed = __any_sync(0xFFFFFFFFu, mixed);
+    __syncwarp();
+  }
   struct Rows {  // one rebuilt input row as the lane sees it
     Frag<T, V> c, c2;
     Frag<T, EW> e;
@@ -170,6 +231,74 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
       const Frag<T, EW> el = combine(IC<EW>{}, ze, ecol);
       const Frag<T, EW> eb = Frag<T, EW>::splat(emode == 1 ? r.c.get(0) : r.c.get(V - 1));
       r.e = emode == 0 ? el : eb;
+    } else if constexpr (CHKF) {
+      const int y = rec.y, ym = rc_ym(rec.info), sc = rc_slot_a(rec.info);
+      const float* wtab = reinterpret_cast<const float*>(ctab);
+      auto chk = [&](auto nc, int gxm, int col) {
+        constexpr int N = decltype(nc)::value;
+        int t = gxm + ym;
+        if (t >= m.den) t -= m.den;
+        const bool kept = m.phase_kept(t);
+        const int da = m.dlo(t), db = m.dhi(t);
+        const int ya = y - da, yb = y + db;
+        const bool ha = ya >= rp.lim_lo, hb = yb <= rp.lim_hi;
+        int sa = (ya - rp.lo) & (p.nr - 1), sb = (yb - rp.lo) & (p.nr - 1);
+        if (!(RECON == R_LI && ha && hb)) {  // nearest loaded row (ties: the lower one)
+          const int s1 = (!hb || (ha && da <= db)) ? sa : sb;
+          sa = s1;
+          sb = s1;
+        }
+        if (kept) {
+          sa = sc;
+          sb = sc;
+        }
+        const Frag<float, N> A = ldf<float, N>(reinterpret_cast<const float*>(ring) + sa * slot_elems + col);
+        if constexpr (RECON == R_NN) {
+          return A;
+        } else {
+          const Frag<float, N> B = ldf<float, N>(reinterpret_cast<const float*>(ring) + sb * slot_elems + col);
+          return lerp_frag<N>(A, B, wtab[t]);
+        }
+      };
+      r.c = chk(IC<V>{}, cc.gxm, ccol);
+      const Frag<T, EW> el = chk(IC<EW>{}, ce.gxm, ecol);
+      const Frag<T, EW> eb = Frag<T, EW>::splat(emode == 1 ? r.c.get(0) : r.c.get(V - 1));
+      r.e = emode == 0 ? el : eb;
+      if constexpr (App::NIN > 1) r.c2 = rebuild_frag<T, V, SCHEME, RECON>(p, m, rp, rec, cc, ring2, slot_elems, ccol, xc, base);
+    } else if constexpr (COLF) {
+      const float* row = reinterpret_cast<const float*>(ring) + rc_slot_a(rec.info) * slot_elems;
+      auto colrow = [&](auto nc, const ColF& z, int col, const float4* wt) {
+        constexpr int N = decltype(nc)::value;
+        const Frag<float, N> c = ldf<float, N>(row + col);
+        const float a = row[z.ca], b = row[z.cb];
+        Frag<float, N> o;
+        if constexpr (RECON == R_LI) {
+          float w[8];
+          const float4 w0 = wt[0];
+          w[0] = w0.x; w[1] = w0.y; w[2] = w0.z; w[3] = w0.w;
+          if constexpr (N > 4) {
+            const float4 w1 = wt[32];
+            w[4] = w1.x; w[5] = w1.y; w[6] = w1.z; w[7] = w1.w;
+          }
+          const float d = a - b;
+#pragma unroll
+          for (int i = 0; i < N; ++i) o.v[i] = z.kept ? c.v[i] : fmaf(d, w[i], b);
+        } else {
+          if (nn_mixed) {
+#pragma unroll
+            for (int i = 0; i < N; ++i) o.v[i] = z.kept ? c.v[i] : (2 * i <= z.lim ? a : b);
+          } else {
+#pragma unroll
+            for (int i = 0; i < N; ++i) o.v[i] = z.kept ? c.v[i] : a;
+          }
+        }
+        return o;
+      };
+      r.c = colrow(IC<V>{}, fc, ccol, ctab + lane);
+      const Frag<T, EW> el = colrow(IC<EW>{}, fe, ecol, ctab + 64 + lane);
+      const Frag<T, EW> eb = Frag<T, EW>::splat(emode == 1 ? r.c.get(0) : r.c.get(V - 1));
+      r.e = emode == 0 ? el : eb;
+      if constexpr (App::NIN > 1) r.c2 = rebuild_frag<T, V, SCHEME, RECON>(p, m, rp, rec, cc, ring2, slot_elems, ccol, xc, base);
     } else if (FAST) {
       r.c = rebuild_frag<T, V, SCHEME, RECON>(p, m, rp, rec, cc, ring, slot_elems, ccol, xc, base);
       if (App::NIN > 1) r.c2 = rebuild_frag<T, V, SCHEME, RECON>(p, m, rp, rec, cc, ring2, slot_elems, ccol, xc, base);
@@ -273,16 +402,18 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
 template <class App, int SCHEME, int RECON, int NCW>
 __device__ __forceinline__ void consumer_fast(const KParams& p, const Mask& m, const RowPlan& rp, int x0, int frame,
                                               int ys, int ye, int g0, uint32_t full_u32, uint32_t empty_u32,
-                                              const typename App::T* ring, int slot_elems, const Recipe* rtab) {
+                                              const typename App::T* ring, int slot_elems, const Recipe* rtab,
+                                              float4* ctab) {
   consumer<App, SCHEME, RECON, NCW, true>(p, m, rp, x0, frame, ys, ye, g0, full_u32, empty_u32, ring, slot_elems,
-                                          rtab);
+                                          rtab, ctab);
 }
 template <class App, int SCHEME, int RECON, int NCW>
 __device__ __noinline__ void consumer_generic(const KParams& p, const Mask& m, const RowPlan& rp, int x0, int frame,
                                               int ys, int ye, int g0, uint32_t full_u32, uint32_t empty_u32,
-                                              const typename App::T* ring, int slot_elems, const Recipe* rtab) {
+                                              const typename App::T* ring, int slot_elems, const Recipe* rtab,
+                                              float4* ctab) {
   consumer<App, SCHEME, RECON, NCW, false>(p, m, rp, x0, frame, ys, ye, g0, full_u32, empty_u32, ring, slot_elems,
-                                           rtab);
+                                           rtab, ctab);
 }
 
 // Persistent CTAs: CTA b processes work items b, b + gridDim.x, ...; an item is
@@ -300,8 +431,10 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : App:
   const int slot_elems = p.row_elems * App::NIN;
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   const int nrec = p.nrec;
-  Recipe* rtab = reinterpret_cast<Recipe*>(smem + bar_bytes + (size_t)p.nr * slot_elems * sizeof(T)) +
-                 max(warp - (p.inline_prod ? 0 : 1), 0) * nrec;  // one recipe table per consumer warp
+  Recipe* rtab0 = reinterpret_cast<Recipe*>(smem + bar_bytes + (size_t)p.nr * slot_elems * sizeof(T));
+  Recipe* rtab = rtab0 + max(warp - (p.inline_prod ? 0 : 1), 0) * nrec;  // one recipe table per consumer warp
+  // column scheme (fp32): per-lane LI weight table, 3 x 32 float4 per consumer warp (kperf.cu: kColTabBytes)
+  float4* ctab = reinterpret_cast<float4*>(rtab0 + NCW * nrec) + max(warp - (p.inline_prod ? 0 : 1), 0) * 96;
   const Mask m{p.num, p.den, p.keep_one};
   const int n_items = p.n_strips * p.n_segs * p.frames;
 
@@ -354,10 +487,10 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : App:
       const bool edges_ok = (exr + App::EW <= p.W) || (exr == p.W);
       if (p.fast_ok && xw + 32 * V <= p.W && edges_ok)
         consumer_fast<App, SCHEME, RECON, NCW>(p, m, rp, x0, frame, ys, ye, g0, full_u32, empty_u32, ring,
-                                               slot_elems, rtab);
+                                               slot_elems, rtab, ctab);
       else
         consumer_generic<App, SCHEME, RECON, NCW>(p, m, rp, x0, frame, ys, ye, g0, full_u32, empty_u32, ring,
-                                                  slot_elems, rtab);
+                                                  slot_elems, rtab, ctab);
     }
   }
 }
