@@ -132,6 +132,10 @@ perf_status perf_run(perf_plan_t plan, const void* in, void* out, void* stream);
  * runs, copies out -> host, synchronises `stream`.  The plan owns the device
  * staging buffers. */
 perf_status perf_run_host(perf_plan_t plan, const void* host_in, void* host_out, void* stream);
+/* (Pipelined: the batch is cut into <= 16 row chunks; chunk i is copied in on a
+ * plan-owned stream, the output rows it completes are computed on `stream`, and
+ * copied out on a second plan-owned stream, so both PCIe directions and the
+ * kernels overlap.  Host buffers should be pinned for the copies to overlap.) */
 
 /* ITERS Hotspot steps on device buffers of W * H floats (a band of H rows
  * starting at global row BAND_Y0 of a GLOBAL_H-row grid when sharded).  T and

@@ -433,8 +433,10 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : App:
   const int nrec = p.nrec;
   Recipe* rtab0 = reinterpret_cast<Recipe*>(smem + bar_bytes + (size_t)p.nr * slot_elems * sizeof(T));
   Recipe* rtab = rtab0 + max(warp - (p.inline_prod ? 0 : 1), 0) * nrec;  // one recipe table per consumer warp
-  // column scheme (fp32): per-lane LI weight table, 3 x 32 float4 per consumer warp (kperf.cu: kColTabBytes)
-  float4* ctab = reinterpret_cast<float4*>(rtab0 + NCW * nrec) + max(warp - (p.inline_prod ? 0 : 1), 0) * 96;
+  // per consumer warp: column scheme (fp32) LI weight table, 3 x 32 float4;
+  // checkerboard LI: den weights (2 float4); kperf.cu sizes it the same way
+  constexpr int CT = SCHEME == S_COL ? 96 : 2;
+  float4* ctab = reinterpret_cast<float4*>(rtab0 + NCW * nrec) + max(warp - (p.inline_prod ? 0 : 1), 0) * CT;
   const Mask m{p.num, p.den, p.keep_one};
   const int n_items = p.n_strips * p.n_segs * p.frames;
 
@@ -515,8 +517,18 @@ cudaError_t launch_one(const KParams& p, unsigned grid, size_t smem, cudaStream_
   // wave-filling choice below (C2: row 1/2 0.178 -> 0.170 ms, exact 0.193 ->
   // 0.181 ms; tools/sweep_tile_h.py).  Cell loaders, u8, Hotspot and the
   // fused pipeline measured best with the wave-filling choice.
+  // (only when that gives >= 2 CTAs per SM: short launches -- perf_run_host's
+  // row chunks -- take the wave-filling choice)
+  static int n_sms = 0;
+  if (n_sms == 0) {
+    int dev = 0;
+    cudaGetDevice(&dev);
+    cudaDeviceGetAttribute(&n_sms, cudaDevAttrMultiProcessorCount, dev);
+    if (n_sms < 1) n_sms = 1;
+  }
   const bool fixed64 = p.seg_auto && p.loader == L_BULK && App::VR <= 2 && App::NIN == 1 && sizeof(typename App::T) == 4 &&
-                       SCHEME != S_STENCIL1;
+                       SCHEME != S_STENCIL1 &&
+                       (long long)p.n_strips * ((p.y_end - p.y_begin + 63) / 64) * p.frames >= 2LL * n_sms;
   if (fixed64) {
     q.seg_h = 64;
     q.n_segs = (p.y_end - p.y_begin + 63) / 64;
@@ -541,7 +553,9 @@ cudaError_t launch_one(const KParams& p, unsigned grid, size_t smem, cudaStream_
     const int seg_cap = p.seg_h;
     int best_n = (rows + seg_cap - 1) / seg_cap;
     const int th = SCHEME == S_STENCIL1 ? p.tile1_h : 1;  // Stencil1 segments hold whole tiles
-    for (int n = (rows + seg_cap - 1) / seg_cap; n <= (rows + 31) / 32 && n <= 4 * best_n + 64; ++n) {
+    // segments >= 32 rows; >= 16 when 32-row segments cannot fill one wave (short launches)
+    const int min_sh = per_seg * ((rows + 31) / 32) >= slots ? 32 : 16;
+    for (int n = (rows + seg_cap - 1) / seg_cap; n <= (rows + min_sh - 1) / min_sh && n <= 4 * best_n + 64; ++n) {
       const int sh = ((rows + n - 1) / n + th - 1) / th * th;
       const int nn = (rows + sh - 1) / sh;
       const long long items = per_seg * nn;

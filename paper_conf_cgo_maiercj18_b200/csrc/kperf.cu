@@ -65,6 +65,8 @@ static BandLayout band_layout(size_t rows, size_t W) {
   return {arr, 3 * arr + 256};
 }
 
+constexpr int kHostChunks = 16;  // perf_run_host: row chunks per call (copy/compute overlap)
+
 struct perf_plan_s {
   int app, W, H, radius, scheme, recon;
   perf_rate rate;
@@ -76,6 +78,17 @@ struct perf_plan_s {
   void* d_stage_in = nullptr;
   void* d_stage_out = nullptr;
   size_t stage_bytes = 0;
+  // perf_run_host pipeline: copy-in / copy-out streams and per-chunk events
+  cudaStream_t s_in = nullptr, s_out = nullptr;
+  cudaEvent_t ev_start = nullptr, ev_done = nullptr;
+  cudaEvent_t ev_in[kHostChunks] = {}, ev_c[kHostChunks] = {};
+  // ... captured once per (host_in, host_out, staging) into a CUDA graph, so a
+  // call is one graph launch instead of ~7 API calls per chunk
+  cudaStream_t s_cap = nullptr;
+  cudaGraphExec_t g_exec = nullptr;
+  const void* g_in = nullptr;
+  void* g_out = nullptr;
+  void* g_stage = nullptr;
   Band band;
   ncclComm_t comm = nullptr;
   int rank = 0, nranks = 1;
@@ -186,8 +199,9 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   k.nrec = s1 ? seg + (seg / k.tile1_h + 1) * 2 * kp::kMaxVR : seg + 2 * kp::kMaxVR;
   // + the column scheme's per-lane LI weight tables / the checkerboard's LI weights
   // (fp32; kernel.cuh ctab: 3 x 32 float4 per consumer warp)
-  const size_t col_tab =
-      ((scheme == PERF_SCHEME_COL || scheme == PERF_SCHEME_CHECKER) && es == 4) ? (size_t)NCW * 3 * 32 * 16 : 0;
+  size_t col_tab = 0;
+  if (es == 4 && scheme == PERF_SCHEME_COL) col_tab = (size_t)NCW * 96 * 16;
+  if (es == 4 && scheme == PERF_SCHEME_CHECKER && P->recon == PERF_RECON_LINEAR) col_tab = (size_t)NCW * 2 * 16;
   const size_t rec_bytes0 = (size_t)NCW * k.nrec * sizeof(kp::Recipe) + col_tab;
   while (nr > next_pow2(hold + 1) && bar_bytes(nr) + nr * slot_bytes + rec_bytes0 > 200 * 1024) nr >>= 1;
   k.nr = nr;
@@ -306,8 +320,11 @@ perf_status perf_plan(perf_plan_t* plan, perf_app app, int W, int H, int radius,
   return PERF_OK;
 }
 
+static void host_graph_free(perf_plan_s* p);
+
 perf_status perf_plan_set(perf_plan_t p, int key, long long v) {
   if (!p) return fail(PERF_ERR_INVALID_ARG, "plan is NULL");
+  host_graph_free(p);  // a captured perf_run_host pipeline bakes in the plan's launch parameters
   switch (key) {
     case PERF_KEY_BATCH:
       if (v < 1) return fail(PERF_ERR_INVALID_ARG, "BATCH must be >= 1");
@@ -416,11 +433,123 @@ perf_status perf_run(perf_plan_t p, const void* in, void* out, void* stream) {
   return PERF_OK;
 }
 
+static void host_graph_free(perf_plan_s* p) {
+  if (p->g_exec) cudaGraphExecDestroy(p->g_exec);
+  p->g_exec = nullptr;
+  p->g_in = nullptr;
+  p->g_out = nullptr;
+  p->g_stage = nullptr;
+}
+
+static void host_pipe_free(perf_plan_s* p) {
+  host_graph_free(p);
+  if (p->s_cap) cudaStreamDestroy(p->s_cap);
+  p->s_cap = nullptr;
+  for (int i = 0; i < kHostChunks; ++i) {
+    if (p->ev_in[i]) cudaEventDestroy(p->ev_in[i]);
+    if (p->ev_c[i]) cudaEventDestroy(p->ev_c[i]);
+    p->ev_in[i] = p->ev_c[i] = nullptr;
+  }
+  if (p->ev_start) cudaEventDestroy(p->ev_start);
+  if (p->ev_done) cudaEventDestroy(p->ev_done);
+  if (p->s_in) cudaStreamDestroy(p->s_in);
+  if (p->s_out) cudaStreamDestroy(p->s_out);
+  p->ev_start = p->ev_done = nullptr;
+  p->s_in = p->s_out = nullptr;
+}
+
+static cudaError_t host_pipe_init(perf_plan_s* p) {
+  if (p->s_in) return cudaSuccess;
+  cudaError_t e = cudaStreamCreateWithFlags(&p->s_in, cudaStreamNonBlocking);
+  if (e == cudaSuccess) e = cudaStreamCreateWithFlags(&p->s_cap, cudaStreamNonBlocking);
+  if (e == cudaSuccess) e = cudaStreamCreateWithFlags(&p->s_out, cudaStreamNonBlocking);
+  if (e == cudaSuccess) e = cudaEventCreateWithFlags(&p->ev_start, cudaEventDisableTiming);
+  if (e == cudaSuccess) e = cudaEventCreateWithFlags(&p->ev_done, cudaEventDisableTiming);
+  for (int i = 0; i < kHostChunks && e == cudaSuccess; ++i) {
+    e = cudaEventCreateWithFlags(&p->ev_in[i], cudaEventDisableTiming);
+    if (e == cudaSuccess) e = cudaEventCreateWithFlags(&p->ev_c[i], cudaEventDisableTiming);
+  }
+  if (e != cudaSuccess) host_pipe_free(p);
+  return e;
+}
+
+// Host-buffer entry: the batch is cut into row chunks (<= kHostChunks); chunk
+// i is copied in on s_in and, as soon as it has landed, the kernel computes the
+// output rows ending kHostLag rows above its last row (the rows it reads below
+// an output row -- stencil radius <= 3 + rebuild apron <= 2 (den - 1) <= 14 --
+// are then all in), and those rows are copied out on s_out; PCIe copies in
+// both directions overlap each other and the kernels.
+static perf_status host_enqueue(perf_plan_s* p, const void* host_in, void* host_out, cudaStream_t s) {
+  const size_t es = elem_size(p->app);
+  const size_t frame_bytes = (size_t)p->W * p->H * es;
+  // chunks: per frame nc row ranges of >= kMinChunkRows rows
+  constexpr int kMinChunkRows = 64;  // > kHostLag
+  const int B = (int)p->batch, H = p->H;
+  int nc = std::max(1, std::min(kHostChunks / std::max(B, 1), H / kMinChunkRows));
+  if (B > kHostChunks) nc = 1;
+  const int per = (H + nc - 1) / nc;
+  nc = (H + per - 1) / per;
+  const size_t row_bytes = (size_t)p->W * es;
+  CK(cudaEventRecord(p->ev_start, s));  // order after the caller's earlier work on `stream`
+  CK(cudaStreamWaitEvent(p->s_in, p->ev_start, 0));
+  CK(cudaStreamWaitEvent(p->s_out, p->ev_start, 0));
+  constexpr int kHostLag = 24;  // > radius + rebuild apron of every plan (<= 17)
+  // frames beyond kHostChunks chunks reuse events: process in groups
+  for (int f0 = 0; f0 < B; f0 += std::max(1, kHostChunks / nc)) {
+    const int f1 = std::min(B, f0 + std::max(1, kHostChunks / nc));
+    const int n = (f1 - f0) * nc;
+    for (int i = 0; i < n; ++i) {  // copy-in
+      const int f = f0 + i / nc, c = i % nc, r0 = c * per, r1 = std::min(H, r0 + per);
+      const size_t off = (size_t)f * frame_bytes + (size_t)r0 * row_bytes;
+      CK(cudaMemcpyAsync(static_cast<char*>(p->d_stage_in) + off, static_cast<const char*>(host_in) + off,
+                         (size_t)(r1 - r0) * row_bytes, cudaMemcpyHostToDevice, p->s_in));
+      CK(cudaEventRecord(p->ev_in[i], p->s_in));
+    }
+    for (int i = 0; i < n; ++i) {  // compute + copy-out: output rows [r0, r1) lag the input chunk
+      const int f = f0 + i / nc, c = i % nc;
+      const int r0 = c == 0 ? 0 : c * per - kHostLag, r1 = c == nc - 1 ? H : (c + 1) * per - kHostLag;
+      CK(cudaStreamWaitEvent(s, p->ev_in[i], 0));
+      KParams k;
+      unsigned grid;
+      size_t smem;
+      const char* fin = static_cast<const char*>(p->d_stage_in) + (size_t)f * frame_bytes;
+      char* fout = static_cast<char*>(p->d_stage_out) + (size_t)f * frame_bytes;
+      perf_status st = make_params(p, fin, nullptr, fout, 1, 0, 0, H, 0, r0, r1, k, grid, smem);
+      if (st != PERF_OK) return st;
+      cudaError_t e = dispatch(p, k, grid, smem, s);
+      if (e != cudaSuccess) return cuda_fail(e, "perf_run_host launch");
+      CK(cudaEventRecord(p->ev_c[i], s));
+      CK(cudaStreamWaitEvent(p->s_out, p->ev_c[i], 0));
+      const size_t off = (size_t)f * frame_bytes + (size_t)r0 * row_bytes;
+      CK(cudaMemcpyAsync(static_cast<char*>(host_out) + off, static_cast<const char*>(p->d_stage_out) + off,
+                         (size_t)(r1 - r0) * row_bytes, cudaMemcpyDeviceToHost, p->s_out));
+    }
+    if (f1 < B) {  // the next group reuses the events: its copies wait for this group's
+      CK(cudaEventRecord(p->ev_done, p->s_out));
+      CK(cudaStreamWaitEvent(p->s_in, p->ev_done, 0));
+      CK(cudaStreamWaitEvent(s, p->ev_done, 0));
+    }
+  }
+  CK(cudaEventRecord(p->ev_done, p->s_out));
+  CK(cudaStreamWaitEvent(s, p->ev_done, 0));
+  return PERF_OK;
+}
+
+static bool is_pinned(const void* ptr) {
+  cudaPointerAttributes a;
+  if (cudaPointerGetAttributes(&a, ptr) != cudaSuccess) {
+    cudaGetLastError();
+    return false;
+  }
+  return a.type == cudaMemoryTypeHost;
+}
+
 perf_status perf_run_host(perf_plan_t p, const void* host_in, void* host_out, void* stream) {
   if (!p || !host_in || !host_out) return fail(PERF_ERR_INVALID_ARG, "NULL argument");
   if (p->app == PERF_APP_HOTSPOT) return fail(PERF_ERR_UNSUPPORTED, "Hotspot has no host-buffer entry point");
   const size_t bytes = (size_t)p->batch * p->W * p->H * elem_size(p->app);
   if (p->stage_bytes < bytes) {
+    host_graph_free(p);
     if (p->d_stage_in) cudaFree(p->d_stage_in);
     if (p->d_stage_out) cudaFree(p->d_stage_out);
     p->d_stage_in = p->d_stage_out = nullptr;
@@ -429,11 +558,36 @@ perf_status perf_run_host(perf_plan_t p, const void* host_in, void* host_out, vo
       return fail(PERF_ERR_OOM, "staging allocation failed");
     p->stage_bytes = bytes;
   }
+  CK(host_pipe_init(p));
   cudaStream_t s = static_cast<cudaStream_t>(stream);
-  CK(cudaMemcpyAsync(p->d_stage_in, host_in, bytes, cudaMemcpyHostToDevice, s));
-  perf_status st = perf_run(p, p->d_stage_in, p->d_stage_out, stream);
-  if (st != PERF_OK) return st;
-  CK(cudaMemcpyAsync(host_out, p->d_stage_out, bytes, cudaMemcpyDeviceToHost, s));
+  if (!(is_pinned(host_in) && is_pinned(host_out))) {  // pageable: plain enqueue (copies are synchronous anyway)
+    perf_status st = host_enqueue(p, host_in, host_out, s);
+    if (st != PERF_OK) return st;
+    CK(cudaStreamSynchronize(s));
+    return PERF_OK;
+  }
+  if (!(p->g_exec && p->g_in == host_in && p->g_out == host_out && p->g_stage == p->d_stage_in)) {
+    host_graph_free(p);
+    CK(cudaStreamBeginCapture(p->s_cap, cudaStreamCaptureModeRelaxed));
+    perf_status st = host_enqueue(p, host_in, host_out, p->s_cap);
+    cudaGraph_t g = nullptr;
+    cudaError_t e = cudaStreamEndCapture(p->s_cap, &g);
+    if (st != PERF_OK) {
+      if (g) cudaGraphDestroy(g);
+      return st;
+    }
+    if (e != cudaSuccess) return cuda_fail(e, "perf_run_host graph capture");
+    e = cudaGraphInstantiate(&p->g_exec, g, 0);
+    cudaGraphDestroy(g);
+    if (e != cudaSuccess) {
+      p->g_exec = nullptr;
+      return cuda_fail(e, "perf_run_host graph instantiate");
+    }
+    p->g_in = host_in;
+    p->g_out = host_out;
+    p->g_stage = p->d_stage_in;
+  }
+  CK(cudaGraphLaunch(p->g_exec, s));
   CK(cudaStreamSynchronize(s));
   return PERF_OK;
 }
@@ -880,6 +1034,7 @@ perf_status perf_destroy(perf_plan_t p) {
   if (p->d_tmp) cudaFree(p->d_tmp);
   if (p->d_stage_in) cudaFree(p->d_stage_in);
   if (p->d_stage_out) cudaFree(p->d_stage_out);
+  host_pipe_free(p);
   band_free(p);
   if (p->comm) ncclCommDestroy(p->comm);
   delete p;
