@@ -580,12 +580,20 @@ __device__ __forceinline__ ChunkInfo make_chunk(const KParams& p, const Mask& m,
 
 // fast rebuild of N samples at ring column `col` (global column fx), all in one
 // mask cell described by `ci`; row facts from the recipe
-template <typename T, int N, int SCHEME, int RECON>
+// ULI (row scheme, fp32 LI): no kept / interpolated branch -- every row is
+// b + (a - b) * wa with a kept row given slot_a == slot_b (a - b = 0: exact);
+// smaller code for consumers whose unrolled loop overflows the instruction cache
+template <typename T, int N, int SCHEME, int RECON, bool ULI = false>
 __device__ __forceinline__ Frag<T, N> rebuild_frag(const KParams& p, const Mask& m, const RowPlan& rp,
                                                    const Recipe& rec, const ChunkInfo& ci, const T* ring,
                                                    int slot_elems, int col, int fx, int base) {
   const uint32_t info = rec.info;
   if (SCHEME == S_NONE || SCHEME == S_STENCIL1) return ldf<T, N>(ring + rc_slot_a(info) * slot_elems + col);
+  if constexpr (SCHEME == S_ROW && ULI && RECON == R_LI && sizeof(T) == 4) {
+    const Frag<T, N> a = ldf<T, N>(ring + rc_slot_a(info) * slot_elems + col);
+    const Frag<T, N> b = ldf<T, N>(ring + rc_slot_b(info) * slot_elems + col);
+    return lerp_frag<N>(a, b, rec.wa);
+  }
   if (SCHEME == S_ROW) {
     if (RECON == R_NN || rc_kept(info)) return ldf<T, N>(ring + rc_slot_a(info) * slot_elems + col);
     const Frag<T, N> a = ldf<T, N>(ring + rc_slot_a(info) * slot_elems + col);

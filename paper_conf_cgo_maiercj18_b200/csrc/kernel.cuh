@@ -300,10 +300,10 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
       r.e = emode == 0 ? el : eb;
       if constexpr (App::NIN > 1) r.c2 = rebuild_frag<T, V, SCHEME, RECON>(p, m, rp, rec, cc, ring2, slot_elems, ccol, xc, base);
     } else if (FAST) {
-      r.c = rebuild_frag<T, V, SCHEME, RECON>(p, m, rp, rec, cc, ring, slot_elems, ccol, xc, base);
+      r.c = rebuild_frag<T, V, SCHEME, RECON, App::ULI>(p, m, rp, rec, cc, ring, slot_elems, ccol, xc, base);
       if (App::NIN > 1) r.c2 = rebuild_frag<T, V, SCHEME, RECON>(p, m, rp, rec, cc, ring2, slot_elems, ccol, xc, base);
       // edge fragment: loaded (inside the image) or the clamped border sample -- selects, no branch
-      const Frag<T, EW> el = rebuild_frag<T, EW, SCHEME, RECON>(p, m, rp, rec, ce, ring, slot_elems, ecol, ex, base);
+      const Frag<T, EW> el = rebuild_frag<T, EW, SCHEME, RECON, App::ULI>(p, m, rp, rec, ce, ring, slot_elems, ecol, ex, base);
       const Frag<T, EW> eb = Frag<T, EW>::splat(emode == 1 ? r.c.get(0) : r.c.get(V - 1));
       r.e = emode == 0 ? el : eb;
     } else {
