@@ -48,6 +48,7 @@ struct KParams {
   int row_elems;             // TW + 2*hx
   int fast_ok;               // every V-chunk lies in one mask cell (G % V == 0 or row scheme)
   int vec_io;                // W % V == 0 and 16-B aligned buffers
+  int vec32;                 // 32-B aligned lane chunks of the output (256-bit stores)
   int tile1_w, tile1_h;      // Stencil1 work-group tile
   int nrec;                  // recipe-table entries per consumer warp (>= n_recipes of a segment)
   int inline_prod;           // bulk loader issued by consumer warp 0 (no dedicated producer warp)
@@ -278,6 +279,10 @@ __device__ __forceinline__ void producer(const KParams& p, const Mask& m, const 
     if (p.loader == L_BULK) {
       // whole kept row: one TMA-engine bulk copy per input array
       if (lane == 0) {
+#ifdef KPERF_PROBE_NOLOAD  // experiment: the ring protocol without the global loads
+        mbar_arrive(&full[slot]);
+        continue;
+#endif
         const uint32_t b0 = (uint32_t)((cx1 - cx0) * sizeof(T));
         const uint32_t b1 = NIN > 1 ? (uint32_t)((px1 - px0) * sizeof(T)) : 0u;
         mbar_arrive_expect_tx(&full[slot], b0 + b1);

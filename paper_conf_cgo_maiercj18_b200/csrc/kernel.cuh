@@ -11,6 +11,9 @@
 #ifndef KPERF_PIPELINE
 #define KPERF_PIPELINE 0
 #endif
+#ifndef KPERF_ST256
+#define KPERF_ST256 1  // 256-bit output stores (fp32 lanes: 8 samples)
+#endif
 #ifndef KPERF_MINB
 #define KPERF_MINB 0  // 0: per-app App::MINB
 #endif
@@ -334,7 +337,18 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
   const bool peer_seg = App::NIN > 1 && p.halo_rows > 0 && (p.pu || p.pd) &&
                         (ys < p.y_begin + p.halo_rows || ye > p.y_end - p.halo_rows);
   auto store = [&](T* dst, const Frag<T, V>& o) {
-    if (FAST && p.vec_io) {
+#ifdef KPERF_PROBE_NOSTORE  // experiment: outputs computed but (almost) never stored
+    if (p.y_begin != -12345) {
+      float acc = 0.f;
+#pragma unroll
+      for (int i = 0; i < V; ++i) acc += (float)o.get(i);
+      if (acc == 1.2345e-30f) dst[0] = o.get(0);
+      return;
+    }
+#endif
+    if (FAST && KPERF_ST256 && V * sizeof(T) == 32 && p.vec32) {  // xc % V == 0, W % 8 == 0, 32-B base
+      st_global_v8(dst, reinterpret_cast<const uint4*>(&o)[0], reinterpret_cast<const uint4*>(&o)[1]);
+    } else if (FAST && p.vec_io) {
 #pragma unroll
       for (int q = 0; q < (int)(V * sizeof(T)) / 16; ++q) {
         const uint4 u = reinterpret_cast<const uint4*>(&o)[q];

@@ -163,6 +163,9 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   const bool aligned = ((reinterpret_cast<uintptr_t>(in) | reinterpret_cast<uintptr_t>(out) |
                          reinterpret_cast<uintptr_t>(in2)) & 15) == 0;
   k.vec_io = (P->W % CV == 0) && aligned ? 1 : 0;
+  // 256-bit output stores: every lane chunk (V elements, 32 B for fp32) 32-B aligned
+  k.vec32 = k.vec_io && es == 4 && (P->W % 8 == 0) && ((reinterpret_cast<uintptr_t>(out) & 31) == 0) &&
+            (((size_t)P->W * P->H * es) % 32 == 0) ? 1 : 0;
   int loader = (int)P->loader;
   if (loader == kp::L_AUTO) {
     if (!k.vec_io) loader = kp::L_SCALAR;
@@ -655,6 +658,7 @@ static perf_status band_step(perf_plan_s* p, const float* src, float* dst, int s
   k.pu_row0 = p->band.peer_row0[0];
   k.pd_row0 = p->band.peer_row0[1];
   k.halo_rows = hb;
+  if (((reinterpret_cast<uintptr_t>(pu) | reinterpret_cast<uintptr_t>(pd)) & 31) != 0) k.vec32 = 0;
   cudaError_t e = dispatch(p, k, grid, smem, s);
   if (e != cudaSuccess) return cuda_fail(e, "hotspot band launch");
   return PERF_OK;

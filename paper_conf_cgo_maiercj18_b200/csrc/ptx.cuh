@@ -76,6 +76,15 @@ __device__ __forceinline__ void st_global_v4(void* p, uint32_t a, uint32_t b, ui
                : "memory");
 }
 
+// 256-bit store (sm_100: STG.E.ENL2.256): a lane's 32 B in one instruction, so
+// a warp's row chunk (32 lanes x 32 B) is one fully coalesced 1-KB request;
+// two 128-bit stores per lane each wrote half of every 32-B sector.
+__device__ __forceinline__ void st_global_v8(void* p, const uint4& a, const uint4& b) {
+  asm volatile("st.global.L1::no_allocate.v8.b32 [%0], {%1, %2, %3, %4, %5, %6, %7, %8};" ::"l"(p), "r"(a.x),
+               "r"(a.y), "r"(a.z), "r"(a.w), "r"(b.x), "r"(b.y), "r"(b.z), "r"(b.w)
+               : "memory");
+}
+
 // packed fp16x2 min / max (HMNMX2).  Median lanes hold 0x6400|v (fp16 1024+v),
 // which orders the same as u16, so VIMNMX.U16x2 and HMNMX2 are interchangeable.
 __device__ __forceinline__ uint32_t hmin2u(uint32_t a, uint32_t b) {
