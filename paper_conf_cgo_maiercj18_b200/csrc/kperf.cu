@@ -488,7 +488,10 @@ static perf_status host_enqueue(perf_plan_s* p, const void* host_in, void* host_
   // chunks: per frame nc row ranges of >= kMinChunkRows rows
   constexpr int kMinChunkRows = 64;  // > kHostLag
   const int B = (int)p->batch, H = p->H;
-  int nc = std::max(1, std::min(kHostChunks / std::max(B, 1), H / kMinChunkRows));
+  // and >= 2 MB per chunk: small frames (C1's 1 MB) are one chunk each
+  const size_t row_b = (size_t)p->W * es;
+  const int min_rows = std::max(kMinChunkRows, (int)std::min<size_t>((size_t)H, ((size_t)2 << 20) / row_b));
+  int nc = std::max(1, std::min(kHostChunks / std::max(B, 1), H / min_rows));
   if (B > kHostChunks) nc = 1;
   const int per = (H + nc - 1) / nc;
   nc = (H + per - 1) / per;
