@@ -299,6 +299,9 @@ __device__ __forceinline__ void producer(const KParams& p, const Mask& m, const 
       }
       const uint32_t d0 = lane_dst0 + (uint32_t)(slot * slot_elems * (int)sizeof(T));
       const T* s0 = lane_src0 + roff;
+#ifdef KPERF_PROBE_NOLOAD
+      rmask = 0u;
+#endif
 #pragma unroll
       for (int k = 0; k < KMAX; ++k) {
         const uint32_t pk = rmask & onehot[k];

@@ -1,5 +1,5 @@
 """A/B timing of experiment builds of libkperf.so on C2-sized inputs.
-usage: ab.py [--set row|all|col|checker|median|c5] lib1.so [lib2.so ...]
+usage: [AB_KEYS='{"producer": 2}'] ab.py [--set row|all|col|checker|median|c5] lib1.so [lib2.so ...]
 Each library runs in its own process (KPERF_LIB); the libraries alternate
 over ROUNDS rounds and the per-variant median is printed (ms per launch,
 8 x 4096^2 fp32 frames; median: 4 x 8192^2 u8; c5: 16 x 3840x2160)."""
@@ -25,6 +25,7 @@ import json, sys, torch
 sys.path.insert(0, ROOT)
 import paper_conf_cgo_maiercj18_b200 as kp, synth
 vs = json.loads(sys.argv[1])
+KEYS = json.loads(sys.argv[2]) if len(sys.argv) > 2 else {}
 out = {}
 bufs = {}
 def buf(app):
@@ -43,7 +44,7 @@ def buf(app):
 for v in vs:
     app, r, sch, num, den, rc = v
     W, H, B, x, y = buf(app)
-    with kp.Plan(app, W, H, r, sch, (num, den), rc, batch=B) as p:
+    with kp.Plan(app, W, H, r, sch, (num, den), rc, batch=B, **KEYS) as p:
         for _ in range(3): p.run(x, y)
         e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
         e0.record()
@@ -65,7 +66,8 @@ def main():
     for _ in range(rounds):
         for lib in args:
             env = dict(os.environ, KPERF_LIB=os.path.abspath(lib))
-            o = subprocess.run([sys.executable, "-c", CHILD, json.dumps(vs)], env=env, capture_output=True, text=True)
+            o = subprocess.run([sys.executable, "-c", CHILD, json.dumps(vs), os.environ.get("AB_KEYS", "{}")], env=env,
+                               capture_output=True, text=True)
             line = [ln for ln in o.stdout.splitlines() if ln.startswith("AB")]
             if not line:
                 print(lib, "FAILED", o.stderr[-2000:])
