@@ -63,6 +63,7 @@ template <int R>
 struct AppGauss {  // K1 Gaussian, binomial (2R+1)^2, fp32
   using T = float;
   static constexpr bool ULI = KPERF_ULI;
+  static constexpr bool IPROD = true;
   static constexpr int V = 8, EW = 2, VR = R, NIN = 1, NWIN = 2 * R + 1, MINB = 4;
   f2 h[NWIN][V / 2];  // horizontal results, column pairs (FADD2/FFMA2 vertical pass)
   __device__ void init(const KParams&) {}
@@ -93,6 +94,7 @@ template <int R>
 struct AppSobel {  // K5 Sobel, |(Gx, Gy)|, fp32
   using T = float;
   static constexpr bool ULI = KPERF_ULI;
+  static constexpr bool IPROD = true;
   static constexpr int V = 8, EW = 2, VR = R, NIN = 1, NWIN = 2 * R + 1, MINB = R == 1 ? 4 : 3;
   f2 sx[NWIN][V / 2], dx[NWIN][V / 2];  // horizontal smoothing / derivative, column pairs
   __device__ void init(const KParams&) {}
@@ -135,6 +137,7 @@ struct AppSobel {  // K5 Sobel, |(Gx, Gy)|, fp32
 struct AppInversion {  // K2 Inversion, 255 - x
   using T = float;
   static constexpr bool ULI = KPERF_ULI;
+  static constexpr bool IPROD = true;
   static constexpr int V = 8, EW = 2, VR = 0, NIN = 1, NWIN = 1, MINB = 4;
   __device__ void init(const KParams&) {}
   template <int U>
@@ -152,6 +155,7 @@ struct AppInversion {  // K2 Inversion, 255 - x
 struct AppHotspot {
   using T = float;
   static constexpr bool ULI = KPERF_ULI;
+  static constexpr bool IPROD = true;
   static constexpr int V = 8, EW = 2, VR = 1, NIN = 2, NWIN = 3, MINB = 4;
   float tc[3][V], tl[3], tr[3], pc[3][V];
   float sdc, rx1, ry1, rz1, amb;
@@ -201,6 +205,7 @@ struct AppHotspot {
 struct AppGaussSobel {
   using T = float;
   static constexpr bool ULI = KPERF_GS_ULI;  // uniform row LI (engine.cuh rebuild_frag)
+  static constexpr bool IPROD = false;  // PERF_KEY_PRODUCER 2 ignored: a smaller consumer loop (I-cache)
   static constexpr int V = 8, EW = 4, VR = 3, NIN = 1, NWIN = 5, MINB = 3;
   f2 hh[5][V / 2];  // horizontal Gaussian of the last 5 rows, lane columns, pairs
   float he[5];      // the same for the lane's edge column (xc-1 / xc+V)
@@ -300,6 +305,7 @@ __device__ __forceinline__ uint32_t mx2(uint32_t a, uint32_t b) {
 struct AppMedian {
   using T = uint8_t;
   static constexpr bool ULI = KPERF_ULI;
+  static constexpr bool IPROD = true;
   static constexpr int V = 16, EW = 4, VR = 1, NIN = 1, NWIN = 3, MINB = 3;
   static constexpr int NW = V / 2 + 2;  // 16-bit-pair words per row incl. the two halo words
   uint32_t r[3][NW];  // word 0 = (_, col -1), words 1..V/2 = cols 0..V-1, last = (col V, _)

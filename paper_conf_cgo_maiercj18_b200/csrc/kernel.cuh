@@ -53,7 +53,7 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
   constexpr int TW = NCW * 32 * V;
   const int lane = threadIdx.x & 31, w = (threadIdx.x >> 5) - (p.inline_prod ? 0 : 1);
   // inline producer (bulk loader): consumer warp 0 issues the kept rows itself
-  const bool issuer = p.inline_prod && w == 0;
+  const bool issuer = App::IPROD && p.inline_prod && w == 0;
   uint64_t* full_p = reinterpret_cast<uint64_t*>(__cvta_shared_to_generic(full_u32));
   T* ring_w = const_cast<T*>(ring);
   int issued = 0;
@@ -336,7 +336,7 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
   // banded Hotspot: does this segment emit rows the neighbours need?  (CTA-uniform)
   const bool peer_seg = App::NIN > 1 && p.halo_rows > 0 && (p.pu || p.pd) &&
                         (ys < p.y_begin + p.halo_rows || ye > p.y_end - p.halo_rows);
-  auto store = [&](T* dst, const Frag<T, V>& o) {
+  auto store = [&](T* dst, const Frag<T, V>& o) {  // (FAST implies vec_io)
 #ifdef KPERF_PROBE_NOSTORE  // experiment: outputs computed but (almost) never stored
     if (p.y_begin != -12345) {
       float acc = 0.f;
@@ -348,7 +348,7 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
 #endif
     if (FAST && KPERF_ST256 && V * sizeof(T) == 32 && p.vec32) {  // xc % V == 0, W % 8 == 0, 32-B base
       st_global_v8(dst, reinterpret_cast<const uint4*>(&o)[0], reinterpret_cast<const uint4*>(&o)[1]);
-    } else if (FAST && p.vec_io) {
+    } else if (FAST) {
 #pragma unroll
       for (int q = 0; q < (int)(V * sizeof(T)) / 16; ++q) {
         const uint4 u = reinterpret_cast<const uint4*>(&o)[q];
@@ -501,7 +501,7 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : App:
       // either inside or starting exactly at W (then it is the clamped border)
       const int exr = xw + 32 * V;
       const bool edges_ok = (exr + App::EW <= p.W) || (exr == p.W);
-      if (p.fast_ok && xw + 32 * V <= p.W && edges_ok)
+      if (p.fast_ok && p.vec_io && xw + 32 * V <= p.W && edges_ok)
         consumer_fast<App, SCHEME, RECON, NCW>(p, m, rp, x0, frame, ys, ye, g0, full_u32, empty_u32, ring,
                                                slot_elems, rtab, ctab);
       else
@@ -526,6 +526,7 @@ cudaError_t launch_one(const KParams& p, unsigned grid, size_t smem, cudaStream_
   // of row segments so the CTA count fills whole waves of resident CTA slots
   // (occupancy API), discounted by the per-segment halo rows.
   KParams q = p;
+  if (!App::IPROD) q.inline_prod = 0;  // (no inline-producer code in this app's consumer loop)
   // fp32 whole-row (TMA bulk) loaders, one input, radius <= 2: fixed 64-row
   // segments -- several waves of short items balance better than the
   // wave-filling choice below (C2: row 1/2 0.178 -> 0.170 ms, exact 0.193 ->
@@ -554,7 +555,7 @@ cudaError_t launch_one(const KParams& p, unsigned grid, size_t smem, cudaStream_
       int dev = 0;
       cudaGetDevice(&dev);
       cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
-      if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k, 32 * (NCW + (p.inline_prod ? 0 : 1)), smem) !=
+      if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k, 32 * (NCW + (q.inline_prod ? 0 : 1)), smem) !=
               cudaSuccess ||
           per_sm < 1)
         per_sm = 1;
@@ -583,7 +584,7 @@ cudaError_t launch_one(const KParams& p, unsigned grid, size_t smem, cudaStream_
     q.n_segs = (rows + q.seg_h - 1) / q.seg_h;
     grid = (unsigned)((long long)q.n_strips * q.n_segs * q.frames);
   }
-  k<<<grid, 32 * (NCW + (p.inline_prod ? 0 : 1)), smem, s>>>(q);
+  k<<<grid, 32 * (NCW + (q.inline_prod ? 0 : 1)), smem, s>>>(q);
   return cudaGetLastError();
 }
 
