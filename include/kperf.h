@@ -102,7 +102,9 @@ enum {
   PERF_KEY_HALO_ROWS = 11,     /* read-only: rows a Hotspot band exchanges with each neighbour per step */
   PERF_KEY_TILE1_W = 12,       /* STENCIL1 tile width: power of two, 16..256 (fp32) / 16..512 (u8); default 16 */
   PERF_KEY_TILE1_H = 13,       /* STENCIL1 tile height, 1..1024; default 16 */
-  PERF_KEY_PRODUCER = 14,      /* 0 auto = 1 dedicated producer warp; 2 bulk rows issued by consumer warp 0 */
+  PERF_KEY_PRODUCER = 14,      /* 0 auto = 1 dedicated producer warp; 2 bulk rows issued by consumer warp 0
+                                  (only in builds with -DKPERF_IPROD=1; the default build ignores 2: the
+                                  inline-producer code slowed every consumer loop) */
   PERF_KEY_TBLOCK = 15,        /* Hotspot temporal blocking: steps per launch, 1..8 (default 1).  CHANGES
                                   RESULTS: T is loaded (perforated, rebuilt) once per launch and the other
                                   steps of the launch read on-chip T (R19).

@@ -16,6 +16,9 @@
 #ifndef KPERF_ULI
 #define KPERF_ULI 0
 #endif
+#ifndef KPERF_IPROD
+#define KPERF_IPROD 0  // inline producer (PERF_KEY_PRODUCER 2) compiled in: slower and a bigger hot loop
+#endif
 #ifndef KPERF_GS_ULI
 #define KPERF_GS_ULI 1
 #endif
@@ -63,7 +66,7 @@ template <int R>
 struct AppGauss {  // K1 Gaussian, binomial (2R+1)^2, fp32
   using T = float;
   static constexpr bool ULI = KPERF_ULI;
-  static constexpr bool IPROD = true;
+  static constexpr bool IPROD = KPERF_IPROD;
   static constexpr int V = 8, EW = 2, VR = R, NIN = 1, NWIN = 2 * R + 1, MINB = 4;
   f2 h[NWIN][V / 2];  // horizontal results, column pairs (FADD2/FFMA2 vertical pass)
   __device__ void init(const KParams&) {}
@@ -94,7 +97,7 @@ template <int R>
 struct AppSobel {  // K5 Sobel, |(Gx, Gy)|, fp32
   using T = float;
   static constexpr bool ULI = KPERF_ULI;
-  static constexpr bool IPROD = true;
+  static constexpr bool IPROD = KPERF_IPROD;
   static constexpr int V = 8, EW = 2, VR = R, NIN = 1, NWIN = 2 * R + 1, MINB = R == 1 ? 4 : 3;
   f2 sx[NWIN][V / 2], dx[NWIN][V / 2];  // horizontal smoothing / derivative, column pairs
   __device__ void init(const KParams&) {}
@@ -137,7 +140,7 @@ struct AppSobel {  // K5 Sobel, |(Gx, Gy)|, fp32
 struct AppInversion {  // K2 Inversion, 255 - x
   using T = float;
   static constexpr bool ULI = KPERF_ULI;
-  static constexpr bool IPROD = true;
+  static constexpr bool IPROD = KPERF_IPROD;
   static constexpr int V = 8, EW = 2, VR = 0, NIN = 1, NWIN = 1, MINB = 4;
   __device__ void init(const KParams&) {}
   template <int U>
@@ -155,7 +158,7 @@ struct AppInversion {  // K2 Inversion, 255 - x
 struct AppHotspot {
   using T = float;
   static constexpr bool ULI = KPERF_ULI;
-  static constexpr bool IPROD = true;
+  static constexpr bool IPROD = KPERF_IPROD;
   static constexpr int V = 8, EW = 2, VR = 1, NIN = 2, NWIN = 3, MINB = 4;
   float tc[3][V], tl[3], tr[3], pc[3][V];
   float sdc, rx1, ry1, rz1, amb;
@@ -305,7 +308,7 @@ __device__ __forceinline__ uint32_t mx2(uint32_t a, uint32_t b) {
 struct AppMedian {
   using T = uint8_t;
   static constexpr bool ULI = KPERF_ULI;
-  static constexpr bool IPROD = true;
+  static constexpr bool IPROD = KPERF_IPROD;
   static constexpr int V = 16, EW = 4, VR = 1, NIN = 1, NWIN = 3, MINB = 3;
   static constexpr int NW = V / 2 + 2;  // 16-bit-pair words per row incl. the two halo words
   uint32_t r[3][NW];  // word 0 = (_, col -1), words 1..V/2 = cols 0..V-1, last = (col V, _)

@@ -163,6 +163,8 @@ def test_loaders_and_tiles_give_identical_bits():
 
 
 def test_inline_producer_gives_identical_bits():
+    """PERF_KEY_PRODUCER 2 (inline producer in -DKPERF_IPROD=1 builds, ignored
+    otherwise) never changes results."""
     W, H = 2048, 260
     img = synth.image("natural", 19, W, H)
     for scheme, rate, recon in [("row", (1, 2), "li"), ("none", (0, 1), "nn"), ("row", (3, 4), "nn"),
