@@ -17,6 +17,8 @@ SETS = {
                 ("sobel", 1, "checker", 1, 4, "nn")],
     "median": [("median", 1, "none", 0, 1, "nn"), ("median", 1, "col", 1, 2, "nn"), ("median", 1, "row", 1, 2, "nn")],
     "c5": [("gauss_sobel", 2, "none", 0, 1, "nn"), ("gauss_sobel", 2, "row", 1, 2, "li")],
+    "c1": [("gaussian", 2, "none", 0, 1, "nn", 512, 512, 512), ("gaussian", 2, "row", 1, 2, "li", 512, 512, 512),
+           ("sobel", 1, "row", 1, 2, "nn", 512, 512, 512)],
 }
 SETS["all"] = SETS["row"] + SETS["col"] + SETS["checker"]
 
@@ -28,8 +30,10 @@ vs = json.loads(sys.argv[1])
 KEYS = json.loads(sys.argv[2]) if len(sys.argv) > 2 else {}
 out = {}
 bufs = {}
-def buf(app):
-    if app == "median":
+def buf(app, shape=None):
+    if shape:
+        W, H, B = shape; dt = torch.float32
+    elif app == "median":
         W = H = 8192; B = 4; dt = torch.uint8
     elif app == "gauss_sobel":
         W, H, B, dt = 3840, 2160, 16, torch.float32
@@ -42,8 +46,8 @@ def buf(app):
         bufs[k] = (x, torch.empty_like(x))
     return (W, H, B) + bufs[k]
 for v in vs:
-    app, r, sch, num, den, rc = v
-    W, H, B, x, y = buf(app)
+    app, r, sch, num, den, rc = v[:6]
+    W, H, B, x, y = buf(app, v[6:] or None)
     with kp.Plan(app, W, H, r, sch, (num, den), rc, batch=B, **KEYS) as p:
         for _ in range(3): p.run(x, y)
         e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
