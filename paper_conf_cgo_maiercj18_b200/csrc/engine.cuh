@@ -37,6 +37,7 @@ struct KParams {
   void* out;        // frame 0; output row y_global at (y_global - out_row0) * W
   long long in_fstride, out_fstride;
   int W, Hg;                 // width, global height (clamping and mask use global rows)
+  int ncw;                   // consumer warps per CTA (the kernel's NCW; host bookkeeping)
   int in_row0, avail0, avail1, out_row0;
   int y_begin, y_end;        // output rows of this launch (global)
   int num, den, G, keep_one; // skipped fraction num/den, granule G (pixels)

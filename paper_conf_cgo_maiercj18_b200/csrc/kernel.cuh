@@ -433,7 +433,8 @@ __device__ __noinline__ void consumer_generic(const KParams& p, const Mask& m, c
 // Persistent CTAs: CTA b processes work items b, b + gridDim.x, ...; an item is
 // (frame, segment of seg_h output rows, strip of TW columns), strip fastest.
 template <class App, int SCHEME, int RECON, int NCW>
-__global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : App::MINB) perf_kernel(const __grid_constant__ KParams p) {
+__global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : (NCW == 2 ? 6 : App::MINB))
+    perf_kernel(const __grid_constant__ KParams p) {
   using T = typename App::T;
   constexpr int V = App::V;
   constexpr int TW = NCW * 32 * V;
@@ -618,5 +619,11 @@ cudaError_t launch_gsobel(int, int, const KParams&, unsigned, size_t, cudaStream
 cudaError_t launch_inversion(int, int, const KParams&, unsigned, size_t, cudaStream_t);
 
 constexpr int kNCW = 4;  // consumer warps per CTA (tile width 1024 fp32 / 4096 u8 columns)
+// narrow images (fp32 W <= 512, e.g. C1's 512^2 frames): 2 consumer warps per
+// CTA, so no consumer warp idles right of the image (Gaussian / Sobel)
+cudaError_t launch_gauss1_n2(int, int, const KParams&, unsigned, size_t, cudaStream_t);
+cudaError_t launch_gauss2_n2(int, int, const KParams&, unsigned, size_t, cudaStream_t);
+cudaError_t launch_sobel1_n2(int, int, const KParams&, unsigned, size_t, cudaStream_t);
+cudaError_t launch_sobel2_n2(int, int, const KParams&, unsigned, size_t, cudaStream_t);
 
 }  // namespace kp

@@ -130,7 +130,9 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   const int CV = 16 / es;  // elements per 16-B chunk (load / store / alignment unit)
   // elements per consumer lane per row (must match App::V in apps.cuh)
   const int V = P->app == PERF_APP_MEDIAN ? 16 : 8;
-  const int NCW = kp::kNCW;
+  // consumer warps per CTA: 2 for narrow fp32 Gaussian / Sobel images (kernel.cuh)
+  const bool narrow = (P->app == PERF_APP_GAUSSIAN || P->app == PERF_APP_SOBEL) && P->W <= 2 * 32 * V;
+  const int NCW = narrow ? 2 : kp::kNCW;
   const int TW = NCW * 32 * V;
   const int Hg = P->global_h > 0 ? (int)P->global_h : P->H;
   int scheme = P->scheme;
@@ -143,6 +145,7 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   k.in_fstride = (long long)P->W * P->H;
   k.out_fstride = (long long)P->W * P->H;
   k.W = P->W;
+  k.ncw = NCW;
   k.Hg = Hg;
   k.in_row0 = in_row0;
   k.avail0 = avail0;
@@ -228,9 +231,15 @@ static cudaError_t dispatch(const perf_plan_s* P, const KParams& k, unsigned gri
   const int rc = P->recon;
   switch (P->app) {
     case PERF_APP_GAUSSIAN:
+      if (k.ncw == 2)
+        return P->radius == 1 ? kp::launch_gauss1_n2(scheme, rc, k, grid, smem, s)
+                              : kp::launch_gauss2_n2(scheme, rc, k, grid, smem, s);
       return P->radius == 1 ? kp::launch_gauss1(scheme, rc, k, grid, smem, s)
                             : kp::launch_gauss2(scheme, rc, k, grid, smem, s);
     case PERF_APP_SOBEL:
+      if (k.ncw == 2)
+        return P->radius == 1 ? kp::launch_sobel1_n2(scheme, rc, k, grid, smem, s)
+                              : kp::launch_sobel2_n2(scheme, rc, k, grid, smem, s);
       return P->radius == 1 ? kp::launch_sobel1(scheme, rc, k, grid, smem, s)
                             : kp::launch_sobel2(scheme, rc, k, grid, smem, s);
     case PERF_APP_MEDIAN: return kp::launch_median(scheme, rc, k, grid, smem, s);
