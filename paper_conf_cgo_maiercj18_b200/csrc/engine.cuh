@@ -200,8 +200,10 @@ __device__ __forceinline__ RowPlan make_row_plan(const KParams& p, const Mask& m
     r.ord_lo = m.ord(r.lo);
     r.nload = m.ord(r.hi) - r.ord_lo + 1;
   } else if (SCHEME == S_CHECKER) {
-    r.lo = max(ya - (m.den - 1), r.lim_lo);
-    r.hi = min(yb + (m.den - 1), r.lim_hi);
+    // rebuild reach along y: keep-one cells reach den-1 rows, skip-one cells 1 row
+    const int reach = m.keep_one ? m.den - 1 : 1;
+    r.lo = max(ya - reach, r.lim_lo);
+    r.hi = min(yb + reach, r.lim_hi);
     r.ord_lo = r.lo;
     r.nload = r.hi - r.lo + 1;
   } else {
@@ -498,9 +500,10 @@ __device__ __forceinline__ Recipe make_recipe(const KParams& p, const Mask& m, c
       }
     }
   } else if (SCHEME == S_CHECKER) {
+    const int reach = m.keep_one ? m.den - 1 : 1;  // (make_row_plan)
     sa = sb = (y - rp.lo) & nmask;
-    need_hi = min(y + m.den - 1, rp.hi) - rp.lo;
-    need_lo = max(y - (m.den - 1), rp.lo) - rp.lo;
+    need_hi = min(y + reach, rp.hi) - rp.lo;
+    need_lo = max(y - reach, rp.lo) - rp.lo;
   } else {
     sa = sb = (y - rp.lo) & nmask;
     need_hi = need_lo = y - rp.lo;

@@ -193,7 +193,7 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   // ring: rows a consumer holds for reconstruction + prefetch depth
   int hold = 1;
   if (scheme == PERF_SCHEME_ROW) hold = 2;
-  if (scheme == PERF_SCHEME_CHECKER) hold = 2 * k.den - 1;
+  if (scheme == PERF_SCHEME_CHECKER) hold = 2 * (k.keep_one ? k.den - 1 : 1) + 1;  // rows a cell's rebuild spans
   int nr = P->ring > 0 ? next_pow2((int)P->ring) : next_pow2(hold + (hold > 2 ? 4 : 6));
   if (nr < hold + 1) nr = next_pow2(hold + 1);
   const int nin = P->app == PERF_APP_HOTSPOT ? 2 : 1;
