@@ -97,7 +97,9 @@ enum {
   PERF_KEY_TILE_W = 6,         /* consumer warps per CTA (1..8); tile width = warps * 32 * V */
   PERF_KEY_TILE_H = 7,         /* output rows per CTA segment (default 128) */
   PERF_KEY_METRIC = 8,         /* perf_metric used by perf_error (default: MRE; ME for Sobel apps) */
-  PERF_KEY_LOADER = 9,         /* 0 auto, 1 TMA bulk rows, 2 cp.async 16 B, 3 scalar (any alignment) */
+  PERF_KEY_LOADER = 9,         /* 0 auto, 1 TMA bulk rows, 2 cp.async 16 B, 3 scalar (any alignment),
+                                  4 TMA bulk copies of kept cell runs (column / checker, <= 64 cells per tile
+                                  row; never chosen by auto: 2.5x slower than 2 for 128-B cells) */
   PERF_KEY_RING = 10,          /* shared-memory ring depth in rows (0 = auto) */
   PERF_KEY_HALO_ROWS = 11,     /* read-only: rows a Hotspot band exchanges with each neighbour per step */
   PERF_KEY_TILE1_W = 12,       /* STENCIL1 tile width: power of two, 16..256 (fp32) / 16..512 (u8); default 16 */

@@ -29,7 +29,7 @@ namespace kp {
 
 enum { S_NONE = 0, S_ROW = 1, S_COL = 2, S_CHECKER = 3, S_STENCIL1 = 4 };
 enum { R_NN = 0, R_LI = 1 };
-enum { L_AUTO = 0, L_BULK = 1, L_ASYNC16 = 2, L_SCALAR = 3 };
+enum { L_AUTO = 0, L_BULK = 1, L_ASYNC16 = 2, L_SCALAR = 3, L_RUNS = 4 };
 
 struct KParams {
   const void* in;   // frame 0; element (x, y_global) at (y_global - in_row0) * W + x
@@ -279,6 +279,44 @@ __device__ __forceinline__ void producer(const KParams& p, const Mask& m, const 
     const int y = row_of_idx<SCHEME>(m, rp, i);
     const long long roff = (long long)(y - p.in_row0) * p.W;
     T* dst = ring + slot * slot_elems;
+    if (SCHEME == S_COL || SCHEME == S_CHECKER) {
+      if (p.loader == L_RUNS) {
+        // kept cells of the row: one TMA-engine bulk copy per run of consecutive
+        // kept cells (skip-one: up to den-1 cells, keep-one: 1), run starts
+        // spread over the lanes; the row's byte total is armed first
+        const int ym = SCHEME == S_CHECKER ? y % m.den : 0;
+        const int c_lo = cx0 / p.G, c_hi = (cx1 - 1) / p.G;
+        uint32_t bytes = 0;
+        int rs[2], re[2];  // this lane's runs (cells lane, lane + 32 of the row)
+#pragma unroll
+        for (int k = 0; k < 2; ++k) {
+          rs[k] = re[k] = 0;
+          const int c = c_lo + lane + 32 * k;
+          int q = (c + ym) % m.den;
+          const bool start = c <= c_hi && m.phase_kept(q) && (c == c_lo || !m.phase_kept(q == 0 ? m.den - 1 : q - 1));
+          if (start) {
+            int e = c;
+            while (e < c_hi && m.phase_kept((e + 1 + ym) % m.den)) ++e;
+            rs[k] = max(c * p.G, cx0);
+            re[k] = min((e + 1) * p.G, cx1);
+            bytes += (uint32_t)((re[k] - rs[k]) * (int)sizeof(T)) * NIN;
+          }
+        }
+#pragma unroll
+        for (int o = 16; o > 0; o >>= 1) bytes += __shfl_xor_sync(0xFFFFFFFFu, bytes, o);
+        if (lane == 0) mbar_arrive_expect_tx(&full[slot], bytes);
+        __syncwarp();
+#pragma unroll
+        for (int k = 0; k < 2; ++k) {
+          if (re[k] > rs[k]) {
+            const uint32_t b = (uint32_t)((re[k] - rs[k]) * sizeof(T));
+            bulk_g2s(dst + (rs[k] - base), in + roff + rs[k], b, &full[slot]);
+            if (NIN > 1) bulk_g2s(dst + p.row_elems + (rs[k] - base), in2 + roff + rs[k], b, &full[slot]);
+          }
+        }
+        continue;
+      }
+    }
     if (p.loader == L_BULK) {
       // whole kept row: one TMA-engine bulk copy per input array
       if (lane == 0) {

@@ -463,7 +463,7 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : (NCW
   }
   if (threadIdx.x == 0) {
     for (int s = 0; s < p.nr; ++s) {
-      mbar_init(&full[s], p.loader == L_BULK ? 1u : 32u);
+      mbar_init(&full[s], (p.loader == L_BULK || p.loader == L_RUNS) ? 1u : 32u);
       mbar_init(&empty[s], (uint32_t)(32 * nact));  // every consumer lane arrives
     }
     mbar_fence_init();

@@ -65,6 +65,10 @@ static BandLayout band_layout(size_t rows, size_t W) {
   return {arr, 3 * arr + 256};
 }
 
+#ifndef KPERF_RUNS
+#define KPERF_RUNS 0  // auto loader picks TMA bulk runs for column / checker cells (measured 2.5x slower than
+                      // 16-B cp.async: one bulk copy per 128-384-B run makes the TMA unit the bound)
+#endif
 constexpr int kHostChunks = 16;  // perf_run_host: row chunks per call (copy/compute overlap)
 
 struct perf_plan_s {
@@ -169,12 +173,20 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   // 256-bit output stores: every lane chunk (V elements, 32 B for fp32) 32-B aligned
   k.vec32 = k.vec_io && es == 4 && (P->W % 8 == 0) && ((reinterpret_cast<uintptr_t>(out) & 31) == 0) &&
             (((size_t)P->W * P->H * es) % 32 == 0) ? 1 : 0;
+  // TMA bulk runs of kept cells: cells of whole 16-B chunks, <= 64 cells per tile row (2 run slots per lane)
+  const bool runs_ok = k.vec_io && chunk_uniform && (scheme == PERF_SCHEME_COL || scheme == PERF_SCHEME_CHECKER) &&
+                       (TW + 2 * ((CV + k.den * k.G + CV - 1) / CV) * CV) / k.G + 2 <= 64;
   int loader = (int)P->loader;
   if (loader == kp::L_AUTO) {
     if (!k.vec_io) loader = kp::L_SCALAR;
     else if (rowwise) loader = kp::L_BULK;
     else loader = chunk_uniform ? kp::L_ASYNC16 : kp::L_SCALAR;
+    // column / checker cells of >= 16 B: TMA bulk copies of kept cell runs, when
+    // a row's runs fit the producer's 64 run slots (2 per lane)
+    if (loader == kp::L_ASYNC16 && KPERF_RUNS && runs_ok) loader = kp::L_RUNS;
   }
+  if (loader == kp::L_RUNS && !runs_ok)
+    return fail(PERF_ERR_UNSUPPORTED, "loader RUNS needs the column / checker scheme, aligned 16-B cells, <= 64 cells per tile row");
   if (loader == kp::L_BULK && !(k.vec_io && rowwise))
     return fail(PERF_ERR_UNSUPPORTED, "loader BULK needs the row/none scheme, W % V == 0 and 16-B aligned buffers");
   if (loader == kp::L_ASYNC16 && !(k.vec_io && chunk_uniform))
@@ -372,7 +384,7 @@ perf_status perf_plan_set(perf_plan_t p, int key, long long v) {
       p->metric = v;
       return PERF_OK;
     case PERF_KEY_LOADER:
-      if (v < 0 || v > 3) return fail(PERF_ERR_INVALID_ARG, "bad LOADER");
+      if (v < 0 || v > 4) return fail(PERF_ERR_INVALID_ARG, "bad LOADER");
       p->loader = v;
       return PERF_OK;
     case PERF_KEY_RING:

@@ -162,6 +162,22 @@ def test_loaders_and_tiles_give_identical_bits():
                 assert np.array_equal(got, ref), (scheme, ld, th)
 
 
+@pytest.mark.parametrize("scheme,rate,recon", [("col", (1, 2), "li"), ("col", (1, 4), "nn"), ("col", (3, 4), "li"),
+                                                ("checker", (1, 2), "nn"), ("checker", (1, 4), "li"),
+                                                ("checker", (3, 4), "nn")])
+def test_cell_run_loader_gives_identical_bits(scheme, rate, recon):
+    """128-B cells: TMA bulk runs of kept cells (loader 4) == 16-B cp.async
+    (2, the default) == scalar loads (3), bit for bit; and == the oracle."""
+    W, H = 2200, 150  # 3 strips, ragged
+    img = synth.image("natural", 23, W, H)
+    ref = gpu_run("gaussian", 2, img, scheme, rate, recon, G_bytes=128, loader=2)
+    for ld in (0, 3, 4):
+        got = gpu_run("gaussian", 2, img, scheme, rate, recon, G_bytes=128, loader=ld)
+        assert np.array_equal(got, ref), (scheme, rate, recon, ld)
+    want = oracle.run(oracle.params("gaussian", W, H, 2, scheme, rate, recon, 32), img)
+    assert_close("gaussian", 2, ref, want)
+
+
 def test_inline_producer_gives_identical_bits():
     """PERF_KEY_PRODUCER 2 (inline producer in -DKPERF_IPROD=1 builds, ignored
     otherwise) never changes results."""
