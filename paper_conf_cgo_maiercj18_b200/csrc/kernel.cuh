@@ -176,15 +176,28 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
   // checkerboard, fp32: per-lane slot choice instead of a divergent kept /
   // skipped branch; every lane then loads one (NN) or two (LI) ring rows and
   // LI is the row scheme's lerp b + (a - b) * wa (exact when a == b, i.e. for
-  // kept lanes and the NN fallback), wa = db / (da + db) from a per-warp table
-  // (LI only: for NN the old per-lane branch is just one load on either side and
-  // measured faster -- sobel3 checker 1/4 NN 230 -> 252 us with the slot select)
-  constexpr bool CHKF = FAST && SCHEME == S_CHECKER && sizeof(T) == 4 && RECON == R_LI;
+  // kept lanes and the one-sided fallback at the image border).
+  // Everything that depends only on the cell phase t = (gx + y) mod den sits in
+  // a per-warp table of den int4 {da, db, wa bits, NN takes a}: kept phases
+  // have da = db = 0 (the own row), so the per-row work is two ring-slot sums,
+  // two border tests and two selects (KPERF_CHKTAB=0: the former per-row
+  // phase arithmetic, LI only; ~75 -> ~25 integer instructions per warp row)
+#ifndef KPERF_CHKTAB
+#define KPERF_CHKTAB 1
+#endif
+  constexpr bool CHKF = FAST && SCHEME == S_CHECKER && sizeof(T) == 4 && (RECON == R_LI || KPERF_CHKTAB);
   if constexpr (CHKF) {
     if (lane < m.den) {
       const int t = lane;
-      reinterpret_cast<float*>(ctab)[t] =
-          m.phase_kept(t) ? 1.f : __fdiv_rn((float)m.dhi(t), (float)(m.dlo(t) + m.dhi(t)));
+      if (KPERF_CHKTAB) {
+        const bool k = m.phase_kept(t);
+        const int da = k ? 0 : m.dlo(t), db = k ? 0 : m.dhi(t);
+        const float wa = k ? 1.f : __fdiv_rn((float)db, (float)(da + db));
+        reinterpret_cast<int4*>(ctab)[t] = make_int4(da, db, __float_as_int(wa), da <= db ? 1 : 0);
+      } else {
+        reinterpret_cast<float*>(ctab)[t] =
+            m.phase_kept(t) ? 1.f : __fdiv_rn((float)m.dhi(t), (float)(m.dlo(t) + m.dhi(t)));
+      }
     }
     __syncwarp();
   }
@@ -234,6 +247,32 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
       const Frag<T, EW> el = combine(IC<EW>{}, ze, ecol);
       const Frag<T, EW> eb = Frag<T, EW>::splat(emode == 1 ? r.c.get(0) : r.c.get(V - 1));
       r.e = emode == 0 ? el : eb;
+    } else if constexpr (CHKF && KPERF_CHKTAB) {
+      const int y = rec.y, ym = rc_ym(rec.info);
+      const int yr = y - rp.lo, yl = y - rp.lim_lo, yh = rp.lim_hi - y;  // (ring slot of y = yr & nmask)
+      const int4* etab = reinterpret_cast<const int4*>(ctab);
+      const float* ringf = reinterpret_cast<const float*>(ring);
+      auto chk = [&](auto nc, int gxm, int col) {
+        constexpr int N = decltype(nc)::value;
+        int t = gxm + ym;
+        if (t >= m.den) t -= m.den;
+        const int4 e = etab[t];
+        const bool ha = e.x <= yl, hb = e.y <= yh;  // the loaded rows above / below exist
+        const int sa = (yr - e.x) & nmask, sb = (yr + e.y) & nmask;
+        if constexpr (RECON == R_NN) {  // nearest (ties: above); one-sided at the border
+          const int s = (ha && (e.w || !hb)) ? sa : sb;
+          return ldf<float, N>(ringf + s * slot_elems + col);
+        } else {
+          const Frag<float, N> A = ldf<float, N>(ringf + (ha ? sa : sb) * slot_elems + col);
+          const Frag<float, N> B = ldf<float, N>(ringf + (hb ? sb : sa) * slot_elems + col);
+          return lerp_frag<N>(A, B, __int_as_float(e.z));
+        }
+      };
+      r.c = chk(IC<V>{}, cc.gxm, ccol);
+      const Frag<T, EW> el = chk(IC<EW>{}, ce.gxm, ecol);
+      const Frag<T, EW> eb = Frag<T, EW>::splat(emode == 1 ? r.c.get(0) : r.c.get(V - 1));
+      r.e = emode == 0 ? el : eb;
+      if constexpr (App::NIN > 1) r.c2 = rebuild_frag<T, V, SCHEME, RECON>(p, m, rp, rec, cc, ring2, slot_elems, ccol, xc, base);
     } else if constexpr (CHKF) {
       const int y = rec.y, ym = rc_ym(rec.info), sc = rc_slot_a(rec.info);
       const float* wtab = reinterpret_cast<const float*>(ctab);
@@ -449,8 +488,8 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : (NCW
   Recipe* rtab0 = reinterpret_cast<Recipe*>(smem + bar_bytes + (size_t)p.nr * slot_elems * sizeof(T));
   Recipe* rtab = rtab0 + max(warp - (p.inline_prod ? 0 : 1), 0) * nrec;  // one recipe table per consumer warp
   // per consumer warp: column scheme (fp32) LI weight table, 3 x 32 float4;
-  // checkerboard LI: den weights (2 float4); kperf.cu sizes it the same way
-  constexpr int CT = SCHEME == S_COL ? 96 : 2;
+  // checkerboard: den phase entries (8 int4); kperf.cu sizes it the same way
+  constexpr int CT = SCHEME == S_COL ? 96 : 8;
   float4* ctab = reinterpret_cast<float4*>(rtab0 + NCW * nrec) + max(warp - (p.inline_prod ? 0 : 1), 0) * CT;
   const Mask m{p.num, p.den, p.keep_one};
   const int n_items = p.n_strips * p.n_segs * p.frames;

@@ -215,11 +215,11 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   if (s1) seg = (seg + k.tile1_h - 1) / k.tile1_h * k.tile1_h;  // whole Stencil1 tiles per segment
   // recipes per segment: seg + 2 VR rows, Stencil1: every tile restarts its window
   k.nrec = s1 ? seg + (seg / k.tile1_h + 1) * 2 * kp::kMaxVR : seg + 2 * kp::kMaxVR;
-  // + the column scheme's per-lane LI weight tables / the checkerboard's LI weights
+  // + the column scheme's per-lane LI weight tables / the checkerboard's phase table
   // (fp32; kernel.cuh ctab: 3 x 32 float4 per consumer warp)
   size_t col_tab = 0;
   if (es == 4 && scheme == PERF_SCHEME_COL) col_tab = (size_t)NCW * 96 * 16;
-  if (es == 4 && scheme == PERF_SCHEME_CHECKER && P->recon == PERF_RECON_LINEAR) col_tab = (size_t)NCW * 2 * 16;
+  if (es == 4 && scheme == PERF_SCHEME_CHECKER) col_tab = (size_t)NCW * 8 * 16;  // den <= 8 int4 phase entries
   const size_t rec_bytes0 = (size_t)NCW * k.nrec * sizeof(kp::Recipe) + col_tab;
   while (nr > next_pow2(hold + 1) && bar_bytes(nr) + nr * slot_bytes + rec_bytes0 > 200 * 1024) nr >>= 1;
   k.nr = nr;
