@@ -1,5 +1,5 @@
 """A/B timing of experiment builds of libkperf.so on C2-sized inputs.
-usage: [AB_KEYS='{"producer": 2}'] ab.py [--set row|all|col|checker|median|c5] lib1.so [lib2.so ...]
+usage: [AB_KEYS='{"producer": 2}'] ab.py [--set row|all|col|checker|median|c5] lib1.so [lib2.so[@{"ring": 8}] ...]
 Each library runs in its own process (KPERF_LIB); the libraries alternate
 over ROUNDS rounds and the per-variant median is printed (ms per launch,
 8 x 4096^2 fp32 frames; median: 4 x 8192^2 u8; c5: 16 x 3840x2160)."""
@@ -71,8 +71,9 @@ def main():
     res = {lib: [] for lib in args}
     for _ in range(rounds):
         for lib in args:
-            env = dict(os.environ, KPERF_LIB=os.path.abspath(lib))
-            o = subprocess.run([sys.executable, "-c", CHILD, json.dumps(vs), os.environ.get("AB_KEYS", "{}")], env=env,
+            path, _, keys = lib.partition("@")  # lib.so@{"ring": 8}: plan keys for this arm only
+            env = dict(os.environ, KPERF_LIB=os.path.abspath(path))
+            o = subprocess.run([sys.executable, "-c", CHILD, json.dumps(vs), keys or os.environ.get("AB_KEYS", "{}")], env=env,
                                capture_output=True, text=True)
             line = [ln for ln in o.stdout.splitlines() if ln.startswith("AB")]
             if not line:
@@ -81,8 +82,8 @@ def main():
                 continue
             res[lib].append(json.loads(line[0][2:]))
     keys = ["/".join(map(str, v)) for v in vs]
-    print("variant".ljust(30) + "".join(os.path.basename(os.path.dirname(os.path.abspath(l))) [:14].rjust(16)
-                                        + os.path.basename(l)[:10] for l in args))
+    print("variant".ljust(30) + "".join(os.path.basename(l.partition("@")[0])[:12].rjust(14)
+                                        + l.partition("@")[2][:12].ljust(12) for l in args))
     for k in keys:
         row = k.ljust(30)
         for lib in args:
