@@ -46,7 +46,9 @@ struct KParams {
   int seg_auto;              // seg_h is an upper bound; the launcher picks the wave-filling value
   int nr, nr_log2;           // ring slots (power of two)
   int hx;                    // columns of halo/apron each side (multiple of V)
-  int row_elems;             // TW + 2*hx
+  int row_elems;             // TW + 2*hx (slot stride; compact checker: chk_cells * G)
+  int chk_compact;           // keep-one checker: a slot holds only its row's kept cells, cell c at
+                             // ((c - (x0/G - den)) / den) * G (kperf.cu: fast path for every warp)
   int fast_ok;               // every V-chunk lies in one mask cell (G % V == 0 or row scheme)
   int vec_io;                // W % V == 0 and 16-B aligned buffers
   int vec32;                 // 32-B aligned lane chunks of the output (256-bit stores)
@@ -272,6 +274,37 @@ __device__ __forceinline__ void producer(const KParams& p, const Mask& m, const 
   const T* lane_src0 = in + cx0 + lane * V;
   const T* lane_src1 = in2 + cx0 + lane * V;
 
+  // compact keep-one checkerboard slots (kperf.cu chk_compact): a row keeps
+  // cells c == -y mod den only, packed at ((c - (x0/G - den)) / den) * G, so
+  // chunk k has one slot offset for every row that keeps it.  A loop of its
+  // own: the full-width loop below keeps its immediate-offset copies.
+  if constexpr (SCHEME == S_CHECKER && NIN == 1) {
+    if (p.chk_compact && p.loader == L_ASYNC16) {
+      uint32_t coff[KMAX];
+      const int cb = x0 / p.G - m.den;
+#pragma unroll
+      for (int k = 0; k < KMAX; ++k) {
+        const int c = min(cx0 + (lane + 32 * k) * V, cx1 - V);
+        const int cell = c / p.G;
+        coff[k] = (uint32_t)((((cell - cb) / m.den) * p.G + (c - cell * p.G)) * (int)sizeof(T));
+      }
+      const T* s0l = lane_src0;
+      for (int i = 0; i < rp.nload; ++i) {
+        const int g = g0 + i;
+        const int slot = g & (p.nr - 1);
+        if (g >= p.nr) mbar_wait(&empty[slot], ((g >> p.nr_log2) - 1) & 1);
+        const int y = row_of_idx<SCHEME>(m, rp, i);
+        const int ym = y % m.den;
+        const uint32_t rmask = ((kmask >> ym) | (kmask << (m.den - ym))) & dmask;
+        const uint32_t dc = smem_u32(ring) + (uint32_t)(slot * slot_elems * (int)sizeof(T));
+        const T* s0 = s0l + (long long)(y - p.in_row0) * p.W;
+#pragma unroll
+        for (int k = 0; k < KMAX; ++k) cp_async16_if(dc + coff[k], s0 + k * 32 * V, rmask & onehot[k]);
+        cp_async_arrive_noinc(&full[slot]);
+      }
+      return;
+    }
+  }
   for (int i = 0; i < rp.nload; ++i) {
     const int g = g0 + i;
     const int slot = g & (p.nr - 1);

@@ -201,6 +201,22 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
     }
     __syncwarp();
   }
+  // ring columns the checkerboard reads: compact keep-one slots (kperf.cu
+  // chk_compact) hold kept cell c at ((c - (x0/G - den)) / den) * G -- every row
+  // that holds this lane's cell holds it there, so the column is per lane
+  int kcol = ccol, kecol = ecol;
+  if constexpr (CHKF && KPERF_CHKTAB && App::NIN == 1) {
+    if (p.chk_compact) {
+      const int cb = x0 / p.G - m.den;
+      auto cmap = [&](int x) {
+        x = min(max(x, 0), p.W - EW);  // (out-of-image edge fragments: any aligned in-slot column; replaced by the clamp)
+        const int cell = x / p.G;
+        return ((cell - cb) / m.den) * p.G + (x - cell * p.G);
+      };
+      kcol = cmap(xc);
+      kecol = cmap(ex);
+    }
+  }
   ColF fc, fe;
   bool nn_mixed = false;  // some lane's chunk straddles the NN midpoint (G/2 not a multiple of V)
   if constexpr (COLF) {
@@ -268,8 +284,8 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
           return lerp_frag<N>(A, B, __int_as_float(e.z));
         }
       };
-      r.c = chk(IC<V>{}, cc.gxm, ccol);
-      const Frag<T, EW> el = chk(IC<EW>{}, ce.gxm, ecol);
+      r.c = chk(IC<V>{}, cc.gxm, kcol);
+      const Frag<T, EW> el = chk(IC<EW>{}, ce.gxm, kecol);
       const Frag<T, EW> eb = Frag<T, EW>::splat(emode == 1 ? r.c.get(0) : r.c.get(V - 1));
       r.e = emode == 0 ? el : eb;
       if constexpr (App::NIN > 1) r.c2 = rebuild_frag<T, V, SCHEME, RECON>(p, m, rp, rec, cc, ring2, slot_elems, ccol, xc, base);

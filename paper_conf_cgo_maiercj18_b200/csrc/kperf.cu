@@ -65,6 +65,10 @@ static BandLayout band_layout(size_t rows, size_t W) {
   return {arr, 3 * arr + 256};
 }
 
+#ifndef KPERF_CHK_COMPACT
+#define KPERF_CHK_COMPACT 1  // compact keep-one checkerboard ring slots (engine.cuh chk_compact)
+#endif
+static int nin_of(int app) { return app == PERF_APP_HOTSPOT ? 2 : 1; }
 #ifndef KPERF_RUNS
 #define KPERF_RUNS 0  // auto loader picks TMA bulk runs for column / checker cells (measured 2.5x slower than
                       // 16-B cp.async: one bulk copy per 128-384-B run makes the TMA unit the bound)
@@ -202,6 +206,16 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   if (scheme == PERF_SCHEME_COL) hx = ((CV + k.den * k.G + CV - 1) / CV) * CV;
   k.hx = hx;
   k.row_elems = TW + 2 * hx;
+  // keep-one checkerboard (fp32, 16-B cp.async cells, every warp on the fast
+  // path): a row keeps 1 cell in den, so its slot holds only those cells,
+  // packed -- den x smaller slots, the same ring depth
+  k.chk_compact = 0;
+  if (KPERF_CHK_COMPACT && scheme == PERF_SCHEME_CHECKER && k.keep_one && k.den > 1 && es == 4 && nin_of(P->app) == 1 &&
+      loader == kp::L_ASYNC16 && k.fast_ok && k.vec_io && P->W % (32 * V) == 0 && TW % k.G == 0 && hx <= k.G &&
+      (k.G * es) % 16 == 0 && TW + 2 * hx <= 32 * 12 * CV) {
+    k.chk_compact = 1;
+    k.row_elems = ((TW / k.G + k.den + 1) / k.den + 1) * k.G;
+  }
   // ring: rows a consumer holds for reconstruction + prefetch depth
   int hold = 1;
   if (scheme == PERF_SCHEME_ROW) hold = 2;

@@ -162,6 +162,24 @@ def test_loaders_and_tiles_give_identical_bits():
                 assert np.array_equal(got, ref), (scheme, ld, th)
 
 
+@pytest.mark.parametrize("app,r", [("gaussian", 2), ("sobel", 1), ("gaussian", 1)])
+@pytest.mark.parametrize("den", [3, 4, 8])
+@pytest.mark.parametrize("gbytes", [32, 128])
+def test_checker_keep_one_compact_slots(app, r, den, gbytes):
+    """Keep-one checkerboard with W a multiple of the warp width: every warp on
+    the fast path, so the ring slots hold only the row's kept cells (kperf.cu
+    chk_compact).  == the oracle, and bit-identical to the scalar loader
+    (loader 3: full-width slots)."""
+    W, H = 2048, 300  # 2 strips, 3 segments (last ragged)
+    img = synth.image("natural", 41 + den, W, H)
+    for recon in ("nn", "li"):
+        got = gpu_run(app, r, img, "checker", (den - 1, den), recon, G_bytes=gbytes)
+        want = oracle.run(oracle.params(app, W, H, r, "checker", (den - 1, den), recon, gbytes // 4), img)
+        assert_close(app, r, got, want)
+        full = gpu_run(app, r, img, "checker", (den - 1, den), recon, G_bytes=gbytes, loader=3)
+        assert np.array_equal(got, full), (den, recon)
+
+
 @pytest.mark.parametrize("scheme,rate,recon", [("col", (1, 2), "li"), ("col", (1, 4), "nn"), ("col", (3, 4), "li"),
                                                 ("checker", (1, 2), "nn"), ("checker", (1, 4), "li"),
                                                 ("checker", (3, 4), "nn")])
