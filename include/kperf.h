@@ -111,8 +111,20 @@ enum {
                                   RESULTS: T is loaded (perforated, rebuilt) once per launch and the other
                                   steps of the launch read on-chip T (R19).
                                   NONE / ROW schemes; banded plans exchange TBLOCK + den halo rows per launch */
-  PERF_KEY_P2P = 16            /* perf_run_hotspot_bands_local only: 1 = halos by direct peer stores fused into
+  PERF_KEY_P2P = 16,           /* perf_run_hotspot_bands_local only: 1 = halos by direct peer stores fused into
                                   the step kernels + epoch flags (the NEXT-4 path), 0 = device copies */
+  PERF_KEY_CHK_COMPACT = 17,   /* read-only: 1 when perf_run (on aligned buffers) packs keep-one checkerboard
+                                  ring slots with the row's kept cells only */
+  PERF_KEY_OVERLAP = 18,       /* banded Hotspot (NCCL or bands_local): 1 (default) = each launch first computes
+                                  the halo_rows boundary rows at both band edges, then exchanges them on a
+                                  plan-owned stream while the interior rows compute; 0 = one
+                                  whole-band launch, then the exchange.  Same results */
+  PERF_KEY_GRAPH = 19,         /* perf_run_hotspot / bands_local: 1 (default) = the ITERS loop is captured once
+                                  per (buffers, plan state) into a CUDA graph and replayed (one launch per
+                                  call); 0 = eager launches.  Peer-store (P2P) plans always run eagerly.
+                                  Reads 2 after a capture failed and the plan fell back to eager launches */
+  PERF_KEY_EXCHANGE = 20       /* MEASUREMENT ONLY: 0 skips every halo exchange of banded runs (results are
+                                  then wrong at band edges) so the exchange's share of a step can be timed */
 };
 
 /* size of a perf_p2p_export handle */
@@ -164,9 +176,62 @@ perf_status perf_run_hotspot_bands_local(perf_plan_t* plans, int nb, const float
 perf_status perf_error(perf_plan_t plan, const void* exact, const void* approx, void* stream,
                        double* err_out, long long* count_out);
 
-/* Sharded Hotspot: attach an NCCL communicator built from a 128-byte
- * ncclUniqueId (rank, nranks).  Rank k holds global rows
- * [BAND_Y0, BAND_Y0 + H); neighbours exchange loaded halo rows every step. */
+/* Deterministic partial sums of the error metric over BATCH * W * H elements
+ * (device pointers): sums[0] = sum of the per-element terms (|e - a| / |e| over
+ * e != 0 for MRE; |e - a| for ME / MAE), sums[1] = sum |e| (ME), sums[2] =
+ * contributing element count (exact in fp64 below 2^53).  Sums of several
+ * shards add elementwise; perf_error_finish turns them into the metric.
+ * Synchronises `stream`.  (Table 1) */
+perf_status perf_error_sums(perf_plan_t plan, const void* exact, const void* approx, void* stream, double sums[3]);
+/* Host only (no device work): the plan's metric from (summed) partial sums:
+ * MRE = sums[0] / sums[2], ME = sums[0] / sums[1], MAE = sums[0] / sums[2];
+ * 0 when the denominator is 0. */
+perf_status perf_error_finish(perf_plan_t plan, const double sums[3], double* err_out, long long* count_out);
+/* Sharded error: every rank's perf_error_sums are summed
+ * with ncclAllReduce(ncclFloat64, ncclSum) on the plan's communicator
+ * (perf_comm_init), so every rank returns the metric of the whole sharded
+ * batch.  Collective: every rank of the communicator calls it.  Without a
+ * communicator it equals perf_error.  Synchronises `stream`. */
+perf_status perf_error_allreduce(perf_plan_t plan, const void* exact, const void* approx, void* stream,
+                                 double* err_out, long long* count_out);
+
+/* Row-band partition: rank `rank` of `nranks` owns global rows
+ * [BAND_Y0, BAND_Y0 + H) of a GLOBAL_H-row image or grid.  A band buffer holds
+ * one frame as buf_rows = halo_rows + H + halo_rows rows of W elements; buffer
+ * row i is global row BAND_Y0 - halo_rows + i (rows outside the image are
+ * never read).  halo_rows = the rows an output row at a band edge can read
+ * beyond the band: stencil radius (Hotspot: TBLOCK steps of radius 1; the
+ * fused pipeline: 3) plus den for the row and checkerboard schemes (the
+ * rebuild distance of a skipped row, R2).  Each exchange sends
+ * buffer rows [send_up_row, + halo_rows) to up_rank, receives
+ * [recv_up_row, + halo_rows) from it, and likewise with down_rank; a missing
+ * neighbour (grid edge) is -1 and its rows are not exchanged.  Host only. */
+typedef struct {
+  int halo_rows, buf_rows;
+  int up_rank, down_rank;
+  int send_up_row, recv_up_row, send_down_row, recv_down_row;
+} perf_halo_plan;
+perf_status perf_band_halo(perf_plan_t plan, int rank, int nranks, perf_halo_plan* out);
+
+/* One-shot row bands of a BATCH of images (SURVEY 8(e), C2/C3 sharded by rows):
+ * `in_band` holds BATCH frames of perf_band_halo's buf_rows x W elements each
+ * (frame f at f * buf_rows * W), the band's own rows at buffer rows
+ * [halo_rows, halo_rows + H); `out` holds BATCH frames of H x W (the band's
+ * output rows).  With a communicator (perf_comm_init) the halo rows of every
+ * frame are first filled from the neighbouring ranks (one ncclGroup of
+ * ncclSend / ncclRecv on `stream`; every rank calls it, collective); without
+ * one the caller must have filled them.  The mask is anchored to global rows
+ * (R2), so the bands' outputs equal the whole image's rows bit for
+ * bit.  Asynchronous on `stream`.  PERF_ERR_UNSUPPORTED for Hotspot (use
+ * perf_run_hotspot) and for STENCIL1 bands not starting on a tile row. */
+perf_status perf_run_band(perf_plan_t plan, void* in_band, void* out, void* stream);
+
+/* Attach an NCCL communicator built from a 128-byte ncclUniqueId (rank,
+ * nranks) -- collective over the ranks.  Used by the sharded Hotspot (rank k
+ * holds global rows [BAND_Y0, BAND_Y0 + H); neighbours exchange halo rows
+ * every launch), perf_run_band and perf_error_allreduce.  The neighbour
+ * connections are set up here (a tiny warm-up exchange), so later exchanges
+ * can be captured into CUDA graphs. */
 perf_status perf_comm_init(perf_plan_t plan, const void* nccl_unique_id, int rank, int nranks);
 /* Fill a 128-byte buffer with a fresh ncclUniqueId (rank 0 calls this). */
 perf_status perf_comm_unique_id(void* out_128_bytes);

@@ -23,18 +23,24 @@ RECON = {"nn": 0, "li": 1, "linear": 1}
 METRIC = {"mre": 0, "me": 1, "mae": 2}
 KEY = {"batch": 1, "iters": 2, "granule_bytes": 3, "global_h": 4, "band_y0": 5, "tile_w": 6, "tile_h": 7,
        "metric": 8, "loader": 9, "ring": 10, "halo_rows": 11, "tile1_w": 12, "tile1_h": 13, "producer": 14,
-       "tblock": 15, "p2p": 16}
+       "tblock": 15, "p2p": 16, "chk_compact": 17, "overlap": 18, "graph": 19, "exchange": 20}
 STATUS = {0: "PERF_OK", 1: "PERF_ERR_INVALID_ARG", 2: "PERF_ERR_UNSUPPORTED", 3: "PERF_ERR_CUDA",
           4: "PERF_ERR_NCCL", 5: "PERF_ERR_OOM"}
 
 # exported symbols of include/kperf.h (tests check the library exports all of them)
 SYMBOLS = ("perf_plan", "perf_plan_set", "perf_plan_get", "perf_run", "perf_run_host", "perf_run_hotspot",
-           "perf_run_hotspot_bands_local", "perf_error", "perf_comm_init", "perf_comm_unique_id",
+           "perf_run_hotspot_bands_local", "perf_error", "perf_error_sums", "perf_error_finish",
+           "perf_error_allreduce", "perf_band_halo", "perf_run_band", "perf_comm_init", "perf_comm_unique_id",
            "perf_p2p_export", "perf_p2p_attach", "perf_destroy", "perf_last_error", "perf_version")
 
 
 class PerfRate(ctypes.Structure):
     _fields_ = [("num", ctypes.c_int), ("den", ctypes.c_int)]
+
+
+class PerfHaloPlan(ctypes.Structure):
+    _fields_ = [(n, ctypes.c_int) for n in ("halo_rows", "buf_rows", "up_rank", "down_rank", "send_up_row",
+                                            "recv_up_row", "send_down_row", "recv_down_row")]
 
 
 class PerfError(RuntimeError):
@@ -63,6 +69,12 @@ def lib():
             "perf_run_hotspot": [vp, vp, vp, vp, vp],
             "perf_run_hotspot_bands_local": [ctypes.POINTER(vp), i, vp, vp, vp, vp],
             "perf_error": [vp, vp, vp, vp, ctypes.POINTER(ctypes.c_double), ctypes.POINTER(ll)],
+            "perf_error_sums": [vp, vp, vp, vp, ctypes.POINTER(ctypes.c_double)],
+            "perf_error_finish": [vp, ctypes.POINTER(ctypes.c_double), ctypes.POINTER(ctypes.c_double),
+                                  ctypes.POINTER(ll)],
+            "perf_error_allreduce": [vp, vp, vp, vp, ctypes.POINTER(ctypes.c_double), ctypes.POINTER(ll)],
+            "perf_band_halo": [vp, i, i, ctypes.POINTER(PerfHaloPlan)],
+            "perf_run_band": [vp, vp, vp, vp],
             "perf_comm_init": [vp, vp, i, i],
             "perf_comm_unique_id": [vp],
             "perf_p2p_export": [vp, vp],
@@ -96,6 +108,35 @@ def _ptr(x) -> int:
     if hasattr(x, "ctypes"):    # numpy array (host buffers for perf_run_host)
         return x.ctypes.data
     raise TypeError(f"cannot take a pointer of {type(x)}")
+
+
+def _check_buf(x, app, numel, device, name):
+    """Argument checks before a pointer crosses the C ABI: dense, the plan's
+    element type, on the right side of the bus, exactly W*H*BATCH elements
+    (the ABI takes bare pointers and cannot check any of this)."""
+    if x is None or isinstance(x, int):
+        return  # raw pointers: the caller's contract (include/kperf.h)
+    want = "uint8" if app == "median" else "float32"
+    if hasattr(x, "data_ptr"):  # torch tensor
+        if not x.is_contiguous():
+            raise ValueError(f"{name}: tensor must be contiguous")
+        if str(x.dtype).replace("torch.", "") != want:
+            raise TypeError(f"{name}: dtype {x.dtype}, plan needs {want}")
+        if (x.device.type == "cuda") != device:
+            raise ValueError(f"{name}: tensor on {x.device}, expected a {'cuda' if device else 'host'} tensor")
+        n = x.numel()
+    elif hasattr(x, "ctypes"):  # numpy array: host memory only
+        if device:
+            raise ValueError(f"{name}: numpy array passed where a device buffer is needed")
+        if not x.flags["C_CONTIGUOUS"]:
+            raise ValueError(f"{name}: array must be C-contiguous")
+        if str(x.dtype) != want:
+            raise TypeError(f"{name}: dtype {x.dtype}, plan needs {want}")
+        n = x.size
+    else:
+        raise TypeError(f"{name}: cannot take a pointer of {type(x)}")
+    if n != numel:
+        raise ValueError(f"{name}: {n} elements, plan needs W*H*BATCH = {numel}")
 
 
 def _stream(stream) -> int:
@@ -157,6 +198,41 @@ def perf_error(plan: int, exact, approx, stream=None):
     return v.value, c.value
 
 
+def perf_error_sums(plan: int, exact, approx, stream=None):
+    """(sum of terms, sum |e|, count) -- shard sums add elementwise"""
+    h = (ctypes.c_double * 3)()
+    _check(lib().perf_error_sums(plan, _ptr(exact), _ptr(approx), _stream(stream), h))
+    return tuple(h)
+
+
+def perf_error_finish(plan: int, sums):
+    """host only: the plan's metric from (summed) partial sums"""
+    h = (ctypes.c_double * 3)(*[float(v) for v in sums])
+    v = ctypes.c_double()
+    c = ctypes.c_longlong()
+    _check(lib().perf_error_finish(plan, h, ctypes.byref(v), ctypes.byref(c)))
+    return v.value, c.value
+
+
+def perf_error_allreduce(plan: int, exact, approx, stream=None):
+    v = ctypes.c_double()
+    c = ctypes.c_longlong()
+    _check(lib().perf_error_allreduce(plan, _ptr(exact), _ptr(approx), _stream(stream), ctypes.byref(v),
+                                      ctypes.byref(c)))
+    return v.value, c.value
+
+
+def perf_band_halo(plan: int, rank: int, nranks: int) -> dict:
+    """host only: the band buffer geometry and halo rows exchanged with each neighbour"""
+    h = PerfHaloPlan()
+    _check(lib().perf_band_halo(plan, rank, nranks, ctypes.byref(h)))
+    return {n: getattr(h, n) for n, _ in PerfHaloPlan._fields_}
+
+
+def perf_run_band(plan: int, in_band, out, stream=None) -> None:
+    _check(lib().perf_run_band(plan, _ptr(in_band), _ptr(out), _stream(stream)))
+
+
 def perf_comm_unique_id() -> bytes:
     buf = ctypes.create_string_buffer(128)
     _check(lib().perf_comm_unique_id(buf))
@@ -207,16 +283,31 @@ class Plan:
     def get(self, key):
         return perf_plan_get(self.handle, key)
 
+    def _elems(self):
+        return self.W * self.H * (1 if self.app == "hotspot" else self.get("batch"))
+
     def run(self, inp, out, stream=None):
+        n = self._elems()
+        _check_buf(inp, self.app, n, device=True, name="in")
+        _check_buf(out, self.app, n, device=True, name="out")
         perf_run(self.handle, inp, out, stream)
 
     def run_host(self, host_in, host_out, stream=None):
+        n = self._elems()
+        _check_buf(host_in, self.app, n, device=False, name="host_in")
+        _check_buf(host_out, self.app, n, device=False, name="host_out")
         perf_run_host(self.handle, host_in, host_out, stream)
 
     def hotspot(self, temp_in, power, temp_out, stream=None):
+        n = self._elems()
+        for b, nm in ((temp_in, "temp_in"), (power, "power"), (temp_out, "temp_out")):
+            _check_buf(b, "hotspot", n, device=True, name=nm)
         perf_run_hotspot(self.handle, temp_in, power, temp_out, stream)
 
     def error(self, exact, approx, stream=None):
+        n = self._elems()
+        _check_buf(exact, self.app, n, device=True, name="exact")
+        _check_buf(approx, self.app, n, device=True, name="approx")
         return perf_error(self.handle, exact, approx, stream)
 
     def close(self):

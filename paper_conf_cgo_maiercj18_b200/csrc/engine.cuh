@@ -298,8 +298,13 @@ __device__ __forceinline__ void producer(const KParams& p, const Mask& m, const 
         const uint32_t rmask = ((kmask >> ym) | (kmask << (m.den - ym))) & dmask;
         const uint32_t dc = smem_u32(ring) + (uint32_t)(slot * slot_elems * (int)sizeof(T));
         const T* s0 = s0l + (long long)(y - p.in_row0) * p.W;
+#ifdef KPERF_PROBE_NOLOAD  // experiment: the ring protocol without the global loads
+        const uint32_t rm = 0u;
+#else
+        const uint32_t rm = rmask;
+#endif
 #pragma unroll
-        for (int k = 0; k < KMAX; ++k) cp_async16_if(dc + coff[k], s0 + k * 32 * V, rmask & onehot[k]);
+        for (int k = 0; k < KMAX; ++k) cp_async16_if(dc + coff[k], s0 + k * 32 * V, rm & onehot[k]);
         cp_async_arrive_noinc(&full[slot]);
       }
       return;

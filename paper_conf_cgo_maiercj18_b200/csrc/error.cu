@@ -77,14 +77,32 @@ __global__ void __launch_bounds__(kErrThreads) err_partial(const T* __restrict__
   }
 }
 
-__global__ void err_final(const double* ps, const double* pt, const long long* pc, int nparts, double* out) {
-  if (threadIdx.x == 0 && blockIdx.x == 0) {
-    double s = 0, t = 0;
-    long long c = 0;
-    for (int i = 0; i < nparts; ++i) { s += ps[i]; t += pt[i]; c += pc[i]; }
-    out[0] = s;
-    out[1] = t;
-    out[2] = (double)c;
+// one block: thread t sums partials t, t + 256, ... in index order, then a
+// fixed-order shared-memory tree (deterministic; the former one-thread loop
+// over 3 x 592 partials was a 65-us serial tail)
+__global__ void __launch_bounds__(kErrThreads) err_final(const double* ps, const double* pt, const long long* pc,
+                                                         int nparts, double* out) {
+  __shared__ double ss[kErrThreads], st[kErrThreads];
+  __shared__ long long sc[kErrThreads];
+  double s = 0, t = 0;
+  long long c = 0;
+  for (int i = threadIdx.x; i < nparts; i += kErrThreads) { s += ps[i]; t += pt[i]; c += pc[i]; }
+  ss[threadIdx.x] = s;
+  st[threadIdx.x] = t;
+  sc[threadIdx.x] = c;
+  __syncthreads();
+  for (int k = kErrThreads / 2; k > 0; k >>= 1) {
+    if (threadIdx.x < k) {
+      ss[threadIdx.x] += ss[threadIdx.x + k];
+      st[threadIdx.x] += st[threadIdx.x + k];
+      sc[threadIdx.x] += sc[threadIdx.x + k];
+    }
+    __syncthreads();
+  }
+  if (threadIdx.x == 0) {
+    out[0] = ss[0];
+    out[1] = st[0];
+    out[2] = (double)sc[0];
   }
 }
 
@@ -104,7 +122,7 @@ cudaError_t launch_error(int is_u8, const void* exact, const void* approx, long 
     err_partial<float><<<kErrBlocks, kErrThreads, 0, s>>>(static_cast<const float*>(exact),
                                                           static_cast<const float*>(approx), n, metric, vec, ps,
                                                           pt, pc);
-  err_final<<<1, 32, 0, s>>>(ps, pt, pc, kErrBlocks, out);
+  err_final<<<1, kErrThreads, 0, s>>>(ps, pt, pc, kErrBlocks, out);
   return cudaGetLastError();
 }
 

@@ -249,11 +249,15 @@ __global__ void __launch_bounds__(32 * TB_WARPS, 3) hotspot_tb_kernel(const __gr
 
 // S steps on output rows [y_begin, y_end); returns the launch error
 cudaError_t launch_hotspot_tb(TBParams q, cudaStream_t s) {
-  static bool attr = false;
-  if (!attr) {
+  constexpr int kMaxDev = 64;  // per device: a process may drive several devices
+  static bool attr[kMaxDev] = {};
+  int dev = 0;
+  cudaGetDevice(&dev);
+  if (dev < 0 || dev >= kMaxDev) dev = 0;
+  if (!attr[dev]) {
     cudaError_t e = cudaFuncSetAttribute(hotspot_tb_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, 227 * 1024);
     if (e != cudaSuccess) return e;
-    attr = true;
+    attr[dev] = true;
   }
   const int L = (q.steps + 3) & ~3;
   q.OW = TB_EW - 2 * L;

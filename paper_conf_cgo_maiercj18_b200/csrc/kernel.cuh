@@ -22,6 +22,25 @@ namespace kp {
 
 constexpr int kMaxVR = 3;  // largest vertical radius of an app (recipe table rows = seg_h + 2 VR)
 
+// per-device host caches (a process may drive several devices through one
+// library: kernel attributes, SM counts and occupancy are per device)
+constexpr int kMaxDev = 64;
+inline int cur_dev() {
+  int d = 0;
+  cudaGetDevice(&d);
+  return (d < 0 || d >= kMaxDev) ? 0 : d;
+}
+inline int dev_sms() {
+  static int sms[kMaxDev] = {};
+  const int d = cur_dev();
+  if (sms[d] == 0) {
+    int v = 0;
+    cudaDeviceGetAttribute(&v, cudaDevAttrMultiProcessorCount, d);
+    sms[d] = v < 1 ? 1 : v;
+  }
+  return sms[d];
+}
+
 
 __device__ __forceinline__ void mbar_wait_u32(uint32_t addr, uint32_t parity) {
   // watchdog: a protocol bug traps (launch error) instead of hanging the GPU
@@ -485,8 +504,8 @@ __device__ __noinline__ void consumer_generic(const KParams& p, const Mask& m, c
                                            rtab, ctab);
 }
 
-// Persistent CTAs: CTA b processes work items b, b + gridDim.x, ...; an item is
-// (frame, segment of seg_h output rows, strip of TW columns), strip fastest.
+// One work item per CTA: CTA b processes item b = (frame, segment of seg_h
+// output rows, strip of TW columns), strip fastest (the launcher sizes seg_h).
 template <class App, int SCHEME, int RECON, int NCW>
 __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : (NCW == 2 ? 6 : App::MINB))
     perf_kernel(const __grid_constant__ KParams p) {
@@ -570,13 +589,14 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : (NCW
 template <class App, int SCHEME, int RECON, int NCW>
 cudaError_t launch_one(const KParams& p, unsigned grid, size_t smem, cudaStream_t s) {
   auto k = perf_kernel<App, SCHEME, RECON, NCW>;
-  static bool attr = false;
-  if (!attr) {
+  static bool attr[kMaxDev] = {};
+  const int dev = cur_dev();
+  if (!attr[dev]) {
     cudaError_t e = cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, 227 * 1024);
     if (e != cudaSuccess) return e;
     e = cudaFuncSetAttribute(k, cudaFuncAttributePreferredSharedMemoryCarveout, 100);  // max shared memory
     if (e != cudaSuccess) return e;
-    attr = true;
+    attr[dev] = true;
   }
   // segment height: when not fixed by the caller (seg_auto), choose the number
   // of row segments so the CTA count fills whole waves of resident CTA slots
@@ -590,13 +610,7 @@ cudaError_t launch_one(const KParams& p, unsigned grid, size_t smem, cudaStream_
   // fused pipeline measured best with the wave-filling choice.
   // (only when that gives >= 2 CTAs per SM: short launches -- perf_run_host's
   // row chunks -- take the wave-filling choice)
-  static int n_sms = 0;
-  if (n_sms == 0) {
-    int dev = 0;
-    cudaGetDevice(&dev);
-    cudaDeviceGetAttribute(&n_sms, cudaDevAttrMultiProcessorCount, dev);
-    if (n_sms < 1) n_sms = 1;
-  }
+  const int n_sms = dev_sms();
   const bool fixed64 = p.seg_auto && p.loader == L_BULK && App::VR <= 2 && App::NIN == 1 && sizeof(typename App::T) == 4 &&
                        SCHEME != S_STENCIL1 &&
                        (long long)p.n_strips * ((p.y_end - p.y_begin + 63) / 64) * p.frames >= 2LL * n_sms;
@@ -605,19 +619,17 @@ cudaError_t launch_one(const KParams& p, unsigned grid, size_t smem, cudaStream_
     q.n_segs = (p.y_end - p.y_begin + 63) / 64;
     grid = (unsigned)((long long)q.n_strips * q.n_segs * q.frames);
   } else if (p.seg_auto) {
-    static int per_sm = 0, sms = 0;
-    static size_t per_sm_smem = 0;
-    if (per_sm == 0 || per_sm_smem != smem) {
-      int dev = 0;
-      cudaGetDevice(&dev);
-      cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
+    static int per_sm_c[kMaxDev] = {};
+    static size_t per_sm_smem[kMaxDev] = {};
+    int& per_sm = per_sm_c[dev];
+    if (per_sm == 0 || per_sm_smem[dev] != smem) {
       if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k, 32 * (NCW + (q.inline_prod ? 0 : 1)), smem) !=
               cudaSuccess ||
           per_sm < 1)
         per_sm = 1;
-      per_sm_smem = smem;
+      per_sm_smem[dev] = smem;
     }
-    const long long slots = (long long)per_sm * sms;
+    const long long slots = (long long)per_sm * n_sms;
     const int rows = p.y_end - p.y_begin;
     const long long per_seg = (long long)p.n_strips * p.frames;
     double best = -1.0;

@@ -79,7 +79,9 @@ struct perf_plan_s {
   int app, W, H, radius, scheme, recon;
   perf_rate rate;
   long long batch = 1, iters = 1, granule_bytes = 128, global_h = -1, band_y0 = 0, tile_w = kp::kNCW, tile_h = 0,
-            metric = 0, loader = 0, ring = 0, tile1_w = 16, tile1_h = 16, producer = 0, tblock = 1, p2p = 0;
+            metric = 0, loader = 0, ring = 0, tile1_w = 16, tile1_h = 16, producer = 0, tblock = 1, p2p = 0,
+            overlap = 1, graph = 1, exchange = 1;
+  unsigned long long gen = 0;  // bumped by every perf_plan_set (graph keys)
   double* d_err = nullptr;
   float* d_tmp = nullptr;
   size_t tmp_elems = 0;
@@ -98,6 +100,12 @@ struct perf_plan_s {
   void* g_out = nullptr;
   void* g_stage = nullptr;
   Band band;
+  // banded Hotspot: exchange stream + fork / join events of the overlapped schedule
+  cudaStream_t s_x = nullptr;
+  cudaEvent_t ev_b = nullptr, ev_x = nullptr;
+  // perf_run_hotspot / bands_local: the ITERS loop captured into a CUDA graph
+  cudaGraphExec_t hg_exec = nullptr;
+  std::vector<const void*> hg_key;
   ncclComm_t comm = nullptr;
   int rank = 0, nranks = 1;
 };
@@ -209,12 +217,16 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   // keep-one checkerboard (fp32, 16-B cp.async cells, every warp on the fast
   // path): a row keeps 1 cell in den, so its slot holds only those cells,
   // packed -- den x smaller slots, the same ring depth
+  // (the consumer reads compact columns only through the phase table, KPERF_CHKTAB;
+  // large cells can make the packed slot wider than the full-width one: keep that)
   k.chk_compact = 0;
-  if (KPERF_CHK_COMPACT && scheme == PERF_SCHEME_CHECKER && k.keep_one && k.den > 1 && es == 4 && nin_of(P->app) == 1 &&
-      loader == kp::L_ASYNC16 && k.fast_ok && k.vec_io && P->W % (32 * V) == 0 && TW % k.G == 0 && hx <= k.G &&
-      (k.G * es) % 16 == 0 && TW + 2 * hx <= 32 * 12 * CV) {
+  const int compact_elems = ((TW / k.G + k.den + 1) / k.den + 1) * k.G;
+  if (KPERF_CHK_COMPACT && KPERF_CHKTAB && scheme == PERF_SCHEME_CHECKER && k.keep_one && k.den > 1 && es == 4 &&
+      nin_of(P->app) == 1 && loader == kp::L_ASYNC16 && k.fast_ok && k.vec_io && P->W % (32 * V) == 0 &&
+      TW % k.G == 0 && hx <= k.G && (k.G * es) % 16 == 0 && TW + 2 * hx <= 32 * 12 * CV &&
+      compact_elems < TW + 2 * hx) {
     k.chk_compact = 1;
-    k.row_elems = ((TW / k.G + k.den + 1) / k.den + 1) * k.G;
+    k.row_elems = compact_elems;
   }
   // ring: rows a consumer holds for reconstruction + prefetch depth
   int hold = 1;
@@ -277,10 +289,13 @@ static cudaError_t dispatch(const perf_plan_s* P, const KParams& k, unsigned gri
 }
 
 static int band_halo(const perf_plan_s* p) {
-  // stencil radius 1 per step of a launch (TBLOCK steps under temporal
-  // blocking) + distance to the loaded rows a rebuilt row reads
+  // rows an output row at a band edge reads beyond the band: the stencil's
+  // vertical radius (Hotspot: radius 1 per step of a launch, TBLOCK steps under
+  // temporal blocking; the fused pipeline: 2 + 1) + the distance to the loaded
+  // rows a rebuilt row reads (row / checkerboard: < den)
   const bool vertical = p->rate.num > 0 && (p->scheme == PERF_SCHEME_ROW || p->scheme == PERF_SCHEME_CHECKER);
-  return (int)p->tblock + (vertical ? p->rate.den : 0);
+  const int vr = p->app == PERF_APP_HOTSPOT ? (int)p->tblock : (p->app == PERF_APP_GAUSS_SOBEL ? 3 : p->radius);
+  return vr + (vertical ? p->rate.den : 0);
 }
 
 // temporally blocked Hotspot launch parameters (hotspot_tb.cu) for a plan
@@ -359,10 +374,13 @@ perf_status perf_plan(perf_plan_t* plan, perf_app app, int W, int H, int radius,
 }
 
 static void host_graph_free(perf_plan_s* p);
+static void hotspot_graph_free(perf_plan_s* p);
 
 perf_status perf_plan_set(perf_plan_t p, int key, long long v) {
   if (!p) return fail(PERF_ERR_INVALID_ARG, "plan is NULL");
   host_graph_free(p);  // a captured perf_run_host pipeline bakes in the plan's launch parameters
+  hotspot_graph_free(p);  // ... and so does a captured Hotspot loop
+  ++p->gen;
   switch (key) {
     case PERF_KEY_BATCH:
       if (v < 1) return fail(PERF_ERR_INVALID_ARG, "BATCH must be >= 1");
@@ -407,6 +425,8 @@ perf_status perf_plan_set(perf_plan_t p, int key, long long v) {
       return PERF_OK;
     case PERF_KEY_HALO_ROWS:
       return fail(PERF_ERR_INVALID_ARG, "HALO_ROWS is read-only");
+    case PERF_KEY_CHK_COMPACT:
+      return fail(PERF_ERR_INVALID_ARG, "CHK_COMPACT is read-only");
     case PERF_KEY_TILE1_W: {
       const long long vmax = p->app == PERF_APP_MEDIAN ? 512 : 256;
       if (v < 16 || v > vmax || (v & (v - 1)))
@@ -429,6 +449,18 @@ perf_status perf_plan_set(perf_plan_t p, int key, long long v) {
     case PERF_KEY_P2P:
       if (v < 0 || v > 1) return fail(PERF_ERR_INVALID_ARG, "P2P must be 0 or 1");
       p->p2p = v;
+      return PERF_OK;
+    case PERF_KEY_OVERLAP:
+      if (v < 0 || v > 1) return fail(PERF_ERR_INVALID_ARG, "OVERLAP must be 0 or 1");
+      p->overlap = v;
+      return PERF_OK;
+    case PERF_KEY_GRAPH:
+      if (v < 0 || v > 1) return fail(PERF_ERR_INVALID_ARG, "GRAPH must be 0 or 1");
+      p->graph = v;
+      return PERF_OK;
+    case PERF_KEY_EXCHANGE:
+      if (v < 0 || v > 1) return fail(PERF_ERR_INVALID_ARG, "EXCHANGE must be 0 or 1");
+      p->exchange = v;
       return PERF_OK;
   }
   return fail(PERF_ERR_INVALID_ARG, "unknown key");
@@ -453,6 +485,20 @@ perf_status perf_plan_get(perf_plan_t p, int key, long long* v) {
     case PERF_KEY_PRODUCER: *v = p->producer; return PERF_OK;
     case PERF_KEY_TBLOCK: *v = p->tblock; return PERF_OK;
     case PERF_KEY_P2P: *v = p->p2p; return PERF_OK;
+    case PERF_KEY_OVERLAP: *v = p->overlap; return PERF_OK;
+    case PERF_KEY_GRAPH: *v = p->graph; return PERF_OK;
+    case PERF_KEY_EXCHANGE: *v = p->exchange; return PERF_OK;
+    case PERF_KEY_CHK_COMPACT: {  // the launch geometry perf_run would use on 256-B aligned buffers
+      KParams k;
+      unsigned grid;
+      size_t smem;
+      const void* d = reinterpret_cast<const void*>(uintptr_t(1) << 20);
+      perf_status st = make_params(p, d, nin_of(p->app) > 1 ? d : nullptr, const_cast<void*>(d), (int)p->batch, 0, 0,
+                                   p->H, 0, 0, p->H, k, grid, smem);
+      if (st != PERF_OK) return st;
+      *v = k.chk_compact;
+      return PERF_OK;
+    }
   }
   return fail(PERF_ERR_INVALID_ARG, "unknown key");
 }
@@ -499,7 +545,7 @@ static void host_pipe_free(perf_plan_s* p) {
 static cudaError_t host_pipe_init(perf_plan_s* p) {
   if (p->s_in) return cudaSuccess;
   cudaError_t e = cudaStreamCreateWithFlags(&p->s_in, cudaStreamNonBlocking);
-  if (e == cudaSuccess) e = cudaStreamCreateWithFlags(&p->s_cap, cudaStreamNonBlocking);
+  if (e == cudaSuccess && !p->s_cap) e = cudaStreamCreateWithFlags(&p->s_cap, cudaStreamNonBlocking);
   if (e == cudaSuccess) e = cudaStreamCreateWithFlags(&p->s_out, cudaStreamNonBlocking);
   if (e == cudaSuccess) e = cudaEventCreateWithFlags(&p->ev_start, cudaEventDisableTiming);
   if (e == cudaSuccess) e = cudaEventCreateWithFlags(&p->ev_done, cudaEventDisableTiming);
@@ -663,9 +709,11 @@ static perf_status band_alloc(perf_plan_s* p) {
   return PERF_OK;
 }
 
-// one step of a band: rows [y0, y0+h) of buffer `src` (with halos filled) -> `dst`
-static perf_status band_step(perf_plan_s* p, const float* src, float* dst, int steps, cudaStream_t s,
-                             float* pu = nullptr, float* pd = nullptr) {
+// rows [ya, yb) of one band launch (`steps` Hotspot steps; buffer rows with
+// halos) `src` -> `dst`.  pu / pd: NEXT-4 peer stores of the band's first / last
+// halo rows (whole-band launches only: the kernels key them off y_begin / y_end)
+static perf_status band_launch(perf_plan_s* p, const float* src, float* dst, int steps, int ya, int yb,
+                               cudaStream_t s, float* pu = nullptr, float* pd = nullptr) {
   const int Hg = (int)p->global_h, y0 = (int)p->band_y0, h = p->H, hb = p->band.hb;
   if (p->tblock > 1) {  // `steps` steps in one temporally blocked launch
     kp::TBParams q = tb_params(p, src, p->band.pbuf, dst);
@@ -677,8 +725,8 @@ static perf_status band_step(perf_plan_s* p, const float* src, float* dst, int s
     q.in_row0 = q.out_row0 = y0 - hb;
     q.avail0 = std::max(0, y0 - hb);
     q.avail1 = std::min(Hg, y0 + h + hb);
-    q.y_begin = y0;
-    q.y_end = y0 + h;
+    q.y_begin = ya;
+    q.y_end = yb;
     q.steps = steps;
     cudaError_t e = kp::launch_hotspot_tb(q, s);
     if (e != cudaSuccess) return cuda_fail(e, "hotspot band launch (temporal blocking)");
@@ -688,7 +736,7 @@ static perf_status band_step(perf_plan_s* p, const float* src, float* dst, int s
   unsigned grid;
   size_t smem;
   perf_status st = make_params(p, src, p->band.pbuf, dst, 1, y0 - hb, std::max(0, y0 - hb), std::min(Hg, y0 + h + hb),
-                               y0 - hb, y0, y0 + h, k, grid, smem);
+                               y0 - hb, ya, yb, k, grid, smem);
   if (st != PERF_OK) return st;
   k.in_fstride = k.out_fstride = 0;
   k.pu = pu;
@@ -702,22 +750,48 @@ static perf_status band_step(perf_plan_s* p, const float* src, float* dst, int s
   return PERF_OK;
 }
 
-// NCCL halo exchange of `buf` (rows with halo) between neighbouring bands
-static perf_status band_exchange_nccl(perf_plan_s* p, float* buf, cudaStream_t s) {
-  const int hb = p->band.hb, h = p->H, W = p->W;
-  const size_t n = (size_t)hb * W;
+// the halo rows of a band (perf_band_halo): the single source of the exchange
+// bookkeeping for NCCL, the single-device emulation and the CPU tests
+static perf_halo_plan halo_plan(const perf_plan_s* p, int rank) {
+  perf_halo_plan h;
+  const int hb = band_halo(p), Hg = p->global_h > 0 ? (int)p->global_h : p->H;
+  h.halo_rows = hb;
+  h.buf_rows = p->H + 2 * hb;
+  h.up_rank = p->band_y0 > 0 ? rank - 1 : -1;
+  h.down_rank = p->band_y0 + p->H < Hg ? rank + 1 : -1;
+  h.send_up_row = hb;         // my first hb rows -> the upper band's bottom halo
+  h.recv_up_row = 0;          // its last hb rows -> my top halo
+  h.send_down_row = p->H;     // my last hb rows -> the lower band's top halo
+  h.recv_down_row = p->H + hb;
+  return h;
+}
+
+// NCCL halo exchange: `frames` frames of `frame_elems` elements of `es` bytes,
+// buffer rows as halo_plan() says; one group (all frames, both neighbours)
+static perf_status band_exchange_nccl(perf_plan_s* p, void* buf, size_t es, int frames, size_t frame_elems,
+                                      cudaStream_t s) {
+  if (!p->exchange || !p->comm) return PERF_OK;
+  const perf_halo_plan h = halo_plan(p, p->rank);
+  const size_t W = p->W, row_b = W * es, n = (size_t)h.halo_rows * row_b;
+  char* b = static_cast<char*>(buf);
   if (ncclGroupStart() != ncclSuccess) return fail(PERF_ERR_NCCL, "ncclGroupStart");
-  if (p->rank > 0) {
-    ncclSend(buf + (size_t)hb * W, n, ncclFloat, p->rank - 1, p->comm, s);  // my first rows -> up
-    ncclRecv(buf, n, ncclFloat, p->rank - 1, p->comm, s);                   // its last rows -> my top halo
-  }
-  if (p->rank < p->nranks - 1) {
-    ncclSend(buf + (size_t)h * W, n, ncclFloat, p->rank + 1, p->comm, s);   // my last rows -> down
-    ncclRecv(buf + (size_t)(h + hb) * W, n, ncclFloat, p->rank + 1, p->comm, s);
+  for (int f = 0; f < frames; ++f) {
+    char* fb = b + (size_t)f * frame_elems * es;
+    if (h.up_rank >= 0) {
+      ncclSend(fb + h.send_up_row * row_b, n, ncclUint8, h.up_rank, p->comm, s);
+      ncclRecv(fb + h.recv_up_row * row_b, n, ncclUint8, h.up_rank, p->comm, s);
+    }
+    if (h.down_rank >= 0) {
+      ncclSend(fb + h.send_down_row * row_b, n, ncclUint8, h.down_rank, p->comm, s);
+      ncclRecv(fb + h.recv_down_row * row_b, n, ncclUint8, h.down_rank, p->comm, s);
+    }
   }
   ncclResult_t r = ncclGroupEnd();
   if (r != ncclSuccess) return fail(PERF_ERR_NCCL, std::string("halo exchange: ") + ncclGetErrorString(r));
   return PERF_OK;
+}
+static perf_status band_exchange_f32(perf_plan_s* p, float* buf, cudaStream_t s) {
+  return band_exchange_nccl(p, buf, sizeof(float), 1, 0, s);
 }
 
 // NEXT-4: push my boundary rows of `mine` (buffer rows [hb, 2hb) and [h, h+hb))
@@ -745,6 +819,184 @@ static perf_status p2p_wait(perf_plan_s* p, cudaStream_t s) {
   return e == cudaSuccess ? PERF_OK : cuda_fail(e, "p2p wait");
 }
 
+// exchange stream + fork/join events of the overlapped band schedule
+static cudaError_t xstream_init(perf_plan_s* p) {
+  if (p->s_x) return cudaSuccess;
+  cudaError_t e = cudaStreamCreateWithFlags(&p->s_x, cudaStreamNonBlocking);
+  if (e == cudaSuccess) e = cudaEventCreateWithFlags(&p->ev_b, cudaEventDisableTiming);
+  if (e == cudaSuccess) e = cudaEventCreateWithFlags(&p->ev_x, cudaEventDisableTiming);
+  return e;
+}
+
+// The overlapped launch schedule of one band: rows within
+// halo_rows of either band edge are computed first; their exchange (`xfer`,
+// on the exchange stream) then runs while the interior rows compute; the next
+// launch waits for it.  The interior reads only band rows, so it never waits
+// for a halo.  `split` false: one whole-band launch, then the exchange.
+}  // extern "C" (templates below)
+
+template <class Xfer>
+static perf_status band_launch_overlapped(perf_plan_s* p, const float* src, float* dst, int steps, bool split, bool xchg,
+                                          cudaStream_t s, Xfer&& xfer) {
+  const int y0 = (int)p->band_y0, h = p->H, hb = p->band.hb;
+  perf_status st;
+  if (!split || !xchg) {
+    if ((st = band_launch(p, src, dst, steps, y0, y0 + h, s)) != PERF_OK) return st;
+    return xchg ? xfer(s) : PERF_OK;
+  }
+  if ((st = band_launch(p, src, dst, steps, y0, y0 + hb, s)) != PERF_OK) return st;
+  if ((st = band_launch(p, src, dst, steps, y0 + h - hb, y0 + h, s)) != PERF_OK) return st;
+  CK(cudaEventRecord(p->ev_b, s));
+  CK(cudaStreamWaitEvent(p->s_x, p->ev_b, 0));
+  if ((st = xfer(p->s_x)) != PERF_OK) return st;
+  CK(cudaEventRecord(p->ev_x, p->s_x));
+  if ((st = band_launch(p, src, dst, steps, y0 + hb, y0 + h - hb, s)) != PERF_OK) return st;
+  CK(cudaStreamWaitEvent(s, p->ev_x, 0));
+  return PERF_OK;
+}
+
+extern "C" {
+
+static bool band_splits(const perf_plan_s* p) { return p->overlap && p->H > 2 * band_halo(p); }
+
+// device scratch of perf_run_hotspot (allocated outside any graph capture)
+static perf_status hotspot_prepare(perf_plan_s* p, bool banded) {
+  const long long n = (long long)p->W * p->H;
+  if (!banded && p->iters > 1 && p->tmp_elems < (size_t)n) {
+    if (p->d_tmp) cudaFree(p->d_tmp);
+    p->d_tmp = nullptr;
+    p->tmp_elems = 0;
+    if (cudaMalloc(&p->d_tmp, n * sizeof(float)) != cudaSuccess) return fail(PERF_ERR_OOM, "tmp allocation");
+    p->tmp_elems = n;
+  }
+  if (banded) {
+    perf_status st = band_alloc(p);
+    if (st != PERF_OK) return st;
+    if (p->H < p->band.hb) return fail(PERF_ERR_UNSUPPORTED, "band thinner than its halo");
+    CK(xstream_init(p));
+  }
+  return PERF_OK;
+}
+
+// the whole ITERS loop of perf_run_hotspot, enqueued on `s` (eager or under capture)
+static perf_status hotspot_enqueue(perf_plan_s* p, const float* temp_in, const float* power, float* temp_out,
+                                   cudaStream_t s) {
+  const long long n = (long long)p->W * p->H;
+  const int Hg = p->global_h > 0 ? (int)p->global_h : p->H;
+  const bool banded = Hg != p->H || p->band_y0 != 0;
+  if (!banded && p->tblock > 1) {  // temporal blocking: one launch per TBLOCK steps
+    const long long tb = p->tblock, launches = (p->iters + tb - 1) / tb;
+    const float* src = temp_in;
+    for (long long l = 0; l < launches; ++l) {
+      float* dst = ((launches - 1 - l) % 2 == 0) ? temp_out : p->d_tmp;
+      kp::TBParams q = tb_params(p, src, power, dst);
+      q.vec = q.vec && ((reinterpret_cast<uintptr_t>(temp_in) | reinterpret_cast<uintptr_t>(temp_out) |
+                         reinterpret_cast<uintptr_t>(p->d_tmp)) & 15) == 0;
+      q.steps = (int)std::min(tb, p->iters - l * tb);
+      cudaError_t e = kp::launch_hotspot_tb(q, s);
+      if (e != cudaSuccess) return cuda_fail(e, "hotspot (temporal blocking) launch");
+      src = dst;
+    }
+    return PERF_OK;
+  }
+  if (!banded) {
+    const float* src = temp_in;
+    for (long long i = 0; i < p->iters; ++i) {
+      float* dst = ((p->iters - 1 - i) % 2 == 0) ? temp_out : p->d_tmp;
+      KParams k;
+      unsigned grid;
+      size_t smem;
+      perf_status st = make_params(p, src, power, dst, 1, 0, 0, p->H, 0, 0, p->H, k, grid, smem);
+      if (st != PERF_OK) return st;
+      cudaError_t e = dispatch(p, k, grid, smem, s);
+      if (e != cudaSuccess) return cuda_fail(e, "hotspot launch");
+      src = dst;
+    }
+    return PERF_OK;
+  }
+  // banded: this rank owns global rows [band_y0, band_y0 + H) of Hg
+  const int hb = p->band.hb;
+  const size_t W = p->W;
+  Band& B = p->band;
+  perf_status st;
+  CK(cudaMemcpyAsync(B.buf[0] + hb * W, temp_in, n * sizeof(float), cudaMemcpyDeviceToDevice, s));
+  CK(cudaMemcpyAsync(B.pbuf + hb * W, power, n * sizeof(float), cudaMemcpyDeviceToDevice, s));
+  if (B.p2p) {  // NEXT-4: halos by direct peer stores fused into the step kernels, epoch flags
+    if ((st = p2p_push(p, B.buf[0], B.peer_buf[0][0], B.peer_buf[1][0], s)) != PERF_OK) return st;
+    if ((st = p2p_push(p, B.pbuf, B.peer_pbuf[0], B.peer_pbuf[1], s)) != PERF_OK) return st;
+    if ((st = p2p_signal(p, s)) != PERF_OK || (st = p2p_wait(p, s)) != PERF_OK) return st;
+    int cur = 0;
+    for (long long i = 0; i < p->iters; i += p->tblock) {
+      const int steps = (int)std::min(p->tblock, p->iters - i);
+      if ((st = band_launch(p, B.buf[cur], B.buf[cur ^ 1], steps, (int)p->band_y0, (int)p->band_y0 + p->H, s,
+                            B.peer_buf[0][cur ^ 1], B.peer_buf[1][cur ^ 1])) != PERF_OK)
+        return st;
+      if ((st = p2p_signal(p, s)) != PERF_OK || (st = p2p_wait(p, s)) != PERF_OK) return st;
+      cur ^= 1;
+    }
+    CK(cudaMemcpyAsync(temp_out, B.buf[cur] + hb * W, n * sizeof(float), cudaMemcpyDeviceToDevice, s));
+    return PERF_OK;
+  }
+  // NCCL: P once, T before the first launch, then every launch's boundary rows
+  // overlapped with its interior (band_launch_overlapped); no exchange after the last
+  if ((st = band_exchange_f32(p, B.pbuf, s)) != PERF_OK) return st;
+  if ((st = band_exchange_f32(p, B.buf[0], s)) != PERF_OK) return st;
+  const bool split = band_splits(p);
+  int cur = 0;
+  for (long long i = 0; i < p->iters; i += p->tblock) {
+    const int steps = (int)std::min(p->tblock, p->iters - i);
+    const bool last = i + p->tblock >= p->iters;
+    float* dst = B.buf[cur ^ 1];
+    if ((st = band_launch_overlapped(p, B.buf[cur], dst, steps, split, !last, s,
+                                     [&](cudaStream_t xs) { return band_exchange_f32(p, dst, xs); })) != PERF_OK)
+      return st;
+    cur ^= 1;
+  }
+  CK(cudaMemcpyAsync(temp_out, B.buf[cur] + hb * W, n * sizeof(float), cudaMemcpyDeviceToDevice, s));
+  return PERF_OK;
+}
+
+static void hotspot_graph_free(perf_plan_s* p) {
+  if (p->hg_exec) cudaGraphExecDestroy(p->hg_exec);
+  p->hg_exec = nullptr;
+  p->hg_key.clear();
+}
+
+}  // extern "C" (template below)
+
+// capture `enqueue` (which enqueues on the stream it is given) into the plan's
+// CUDA graph keyed by `key`, then launch it on `s`; on a capture failure fall
+// back to eager launches for this plan (PERF_KEY_GRAPH then reads 2)
+template <class Enq>
+static perf_status graph_run(perf_plan_s* p, const std::vector<const void*>& key, cudaStream_t s, Enq&& enqueue) {
+  if (p->graph != 1) return enqueue(s);
+  if (!(p->hg_exec && p->hg_key == key)) {
+    hotspot_graph_free(p);
+    if (!p->s_cap) CK(cudaStreamCreateWithFlags(&p->s_cap, cudaStreamNonBlocking));
+    CK(cudaStreamBeginCapture(p->s_cap, cudaStreamCaptureModeRelaxed));
+    perf_status st = enqueue(p->s_cap);
+    cudaGraph_t g = nullptr;
+    cudaError_t e = cudaStreamEndCapture(p->s_cap, &g);
+    if (st != PERF_OK) {
+      if (g) cudaGraphDestroy(g);
+      return st;
+    }
+    if (e == cudaSuccess) e = cudaGraphInstantiate(&p->hg_exec, g, 0);
+    if (g) cudaGraphDestroy(g);
+    if (e != cudaSuccess) {  // e.g. a transport that refuses capture: run eagerly from now on
+      cudaGetLastError();
+      p->hg_exec = nullptr;
+      p->graph = 2;
+      return enqueue(s);
+    }
+    p->hg_key = key;
+  }
+  CK(cudaGraphLaunch(p->hg_exec, s));
+  return PERF_OK;
+}
+
+extern "C" {
+
 perf_status perf_run_hotspot(perf_plan_t p, const float* temp_in, const float* power, float* temp_out, void* stream) {
   if (!p || !temp_in || !power || !temp_out) return fail(PERF_ERR_INVALID_ARG, "NULL argument");
   if (p->app != PERF_APP_HOTSPOT) return fail(PERF_ERR_INVALID_ARG, "plan is not a Hotspot plan");
@@ -761,128 +1013,50 @@ perf_status perf_run_hotspot(perf_plan_t p, const float* temp_in, const float* p
     const bool exact = p->rate.num == 0 || p->scheme == PERF_SCHEME_NONE;
     if (!exact && p->scheme != PERF_SCHEME_ROW) return fail(PERF_ERR_UNSUPPORTED, "TBLOCK > 1 needs the NONE or ROW scheme");
   }
-  if (!banded && p->tblock > 1) {  // temporal blocking: one launch per TBLOCK steps
-    const long long tb = p->tblock, launches = (p->iters + tb - 1) / tb;
-    if (launches > 1 && p->tmp_elems < (size_t)n) {
-      if (p->d_tmp) cudaFree(p->d_tmp);
-      p->d_tmp = nullptr;
-      if (cudaMalloc(&p->d_tmp, n * sizeof(float)) != cudaSuccess) return fail(PERF_ERR_OOM, "tmp allocation");
-      p->tmp_elems = n;
-    }
-    const float* src = temp_in;
-    for (long long l = 0; l < launches; ++l) {
-      float* dst = ((launches - 1 - l) % 2 == 0) ? temp_out : p->d_tmp;
-      kp::TBParams q = tb_params(p, src, power, dst);
-      q.vec = q.vec && ((reinterpret_cast<uintptr_t>(temp_in) | reinterpret_cast<uintptr_t>(temp_out) |
-                         reinterpret_cast<uintptr_t>(p->d_tmp)) & 15) == 0;
-      q.steps = (int)std::min(tb, p->iters - l * tb);
-      cudaError_t e = kp::launch_hotspot_tb(q, s);
-      if (e != cudaSuccess) return cuda_fail(e, "hotspot (temporal blocking) launch");
-      src = dst;
-    }
-    return PERF_OK;
-  }
-  if (!banded) {
-    if (p->iters > 1 && p->tmp_elems < (size_t)n) {
-      if (p->d_tmp) cudaFree(p->d_tmp);
-      p->d_tmp = nullptr;
-      if (cudaMalloc(&p->d_tmp, n * sizeof(float)) != cudaSuccess) return fail(PERF_ERR_OOM, "tmp allocation");
-      p->tmp_elems = n;
-    }
-    const float* src = temp_in;
-    for (long long i = 0; i < p->iters; ++i) {
-      float* dst = ((p->iters - 1 - i) % 2 == 0) ? temp_out : p->d_tmp;
-      KParams k;
-      unsigned grid;
-      size_t smem;
-      perf_status st = make_params(p, src, power, dst, 1, 0, 0, p->H, 0, 0, p->H, k, grid, smem);
-      if (st != PERF_OK) return st;
-      cudaError_t e = dispatch(p, k, grid, smem, s);
-      if (e != cudaSuccess) return cuda_fail(e, "hotspot launch");
-      src = dst;
-    }
-    return PERF_OK;
-  }
-  // banded: this rank owns global rows [band_y0, band_y0 + H) of Hg
-  if (!p->comm && !p->band.p2p && p->nranks == 1 && Hg != p->H)
+  if (banded && !p->comm && !p->band.p2p && p->nranks == 1 && Hg != p->H)
     return fail(PERF_ERR_INVALID_ARG,
                 "banded Hotspot needs perf_comm_init or perf_p2p_attach (or perf_run_hotspot_bands_local)");
-  perf_status st = band_alloc(p);
+  perf_status st = hotspot_prepare(p, banded);
   if (st != PERF_OK) return st;
-  const int hb = p->band.hb;
-  if (p->H < hb) return fail(PERF_ERR_UNSUPPORTED, "band thinner than its halo");
-  const size_t W = p->W;
-  CK(cudaMemcpyAsync(p->band.buf[0] + hb * W, temp_in, n * sizeof(float), cudaMemcpyDeviceToDevice, s));
-  CK(cudaMemcpyAsync(p->band.pbuf + hb * W, power, n * sizeof(float), cudaMemcpyDeviceToDevice, s));
-  if (p->band.p2p) {  // NEXT-4: halos by direct peer stores fused into the step kernels, epoch flags
-    Band& B = p->band;
-    if ((st = p2p_push(p, B.buf[0], B.peer_buf[0][0], B.peer_buf[1][0], s)) != PERF_OK) return st;
-    if ((st = p2p_push(p, B.pbuf, B.peer_pbuf[0], B.peer_pbuf[1], s)) != PERF_OK) return st;
-    if ((st = p2p_signal(p, s)) != PERF_OK || (st = p2p_wait(p, s)) != PERF_OK) return st;
-    int cur = 0;
-    for (long long i = 0; i < p->iters; i += p->tblock) {
-      const int steps = (int)std::min(p->tblock, p->iters - i);
-      if ((st = band_step(p, B.buf[cur], B.buf[cur ^ 1], steps, s, B.peer_buf[0][cur ^ 1], B.peer_buf[1][cur ^ 1])) !=
-          PERF_OK)
-        return st;
-      if ((st = p2p_signal(p, s)) != PERF_OK || (st = p2p_wait(p, s)) != PERF_OK) return st;
-      cur ^= 1;
-    }
-    CK(cudaMemcpyAsync(temp_out, B.buf[cur] + hb * W, n * sizeof(float), cudaMemcpyDeviceToDevice, s));
-    return PERF_OK;
-  }
-  if ((st = band_exchange_nccl(p, p->band.pbuf, s)) != PERF_OK) return st;
-  int cur = 0;
-  for (long long i = 0; i < p->iters; i += p->tblock) {  // one halo exchange + launch per TBLOCK steps
-    if ((st = band_exchange_nccl(p, p->band.buf[cur], s)) != PERF_OK) return st;
-    const int steps = (int)std::min(p->tblock, p->iters - i);
-    if ((st = band_step(p, p->band.buf[cur], p->band.buf[cur ^ 1], steps, s)) != PERF_OK) return st;
-    cur ^= 1;
-  }
-  CK(cudaMemcpyAsync(temp_out, p->band.buf[cur] + hb * W, n * sizeof(float), cudaMemcpyDeviceToDevice, s));
-  return PERF_OK;
+  auto enq = [&](cudaStream_t cs) { return hotspot_enqueue(p, temp_in, power, temp_out, cs); };
+  if (banded && p->band.p2p) return enq(s);  // host-side epoch counters: never replayed from a graph
+  return graph_run(p, {temp_in, power, temp_out}, s, enq);
 }
 
 /* Single-device emulation of the sharded Hotspot: nb band plans (consecutive
  * bands of one grid) step in lockstep on `stream`, halos copied device to
- * device instead of NCCL.  temp_in/power/temp_out are whole-grid buffers. */
-perf_status perf_run_hotspot_bands_local(perf_plan_t* plans, int nb, const float* temp_in, const float* power,
-                                         float* temp_out, void* stream) {
-  if (!plans || nb < 1 || !temp_in || !power || !temp_out) return fail(PERF_ERR_INVALID_ARG, "bad arguments");
-  cudaStream_t s = static_cast<cudaStream_t>(stream);
+ * device instead of NCCL (same halo_plan bookkeeping, same overlapped
+ * boundary / interior schedule on the exchange stream of plans[0], same graph
+ * capture).  temp_in/power/temp_out are whole-grid buffers. */
+static perf_status bands_local_enqueue(perf_plan_t* plans, int nb, const float* temp_in, const float* power,
+                                       float* temp_out, cudaStream_t s) {
   const size_t W = plans[0]->W;
   const long long iters = plans[0]->iters;
   for (int b = 0; b < nb; ++b) {
     perf_plan_s* p = plans[b];
-    if (!p || p->app != PERF_APP_HOTSPOT || (size_t)p->W != W || p->iters != iters || p->tblock != plans[0]->tblock)
-      return fail(PERF_ERR_INVALID_ARG, "band plans must be Hotspot plans of one grid (same ITERS, TBLOCK)");
-    if (p->tblock > 1 && p->rate.num > 0 && p->scheme != PERF_SCHEME_ROW && p->scheme != PERF_SCHEME_NONE)
-      return fail(PERF_ERR_UNSUPPORTED, "TBLOCK > 1 needs the NONE or ROW scheme");
-    if (b > 0 && p->band_y0 != plans[b - 1]->band_y0 + plans[b - 1]->H)
-      return fail(PERF_ERR_INVALID_ARG, "bands must be consecutive");
-    perf_status st = band_alloc(p);
-    if (st != PERF_OK) return st;
-    if (p->H < p->band.hb) return fail(PERF_ERR_UNSUPPORTED, "band thinner than its halo");
     const size_t off = (size_t)p->band_y0 * W, n = (size_t)p->H * W, hbw = (size_t)p->band.hb * W;
     CK(cudaMemcpyAsync(p->band.buf[0] + hbw, temp_in + off, n * sizeof(float), cudaMemcpyDeviceToDevice, s));
     CK(cudaMemcpyAsync(p->band.pbuf + hbw, power + off, n * sizeof(float), cudaMemcpyDeviceToDevice, s));
   }
-  auto exchange = [&](int which, bool power_buf) -> perf_status {
+  // band b's halos from its neighbours' boundary rows, rows as halo_plan() says
+  auto exchange = [&](int which, bool power_buf, cudaStream_t xs) -> perf_status {
+    if (!plans[0]->exchange) return PERF_OK;
     for (int b = 0; b < nb; ++b) {
       perf_plan_s* p = plans[b];
+      const perf_halo_plan h = halo_plan(p, b);
       float* mine = power_buf ? p->band.pbuf : p->band.buf[which];
-      const size_t hb = p->band.hb, h = p->H;
-      if (b > 0) {  // top halo <- last hb rows of band b-1
-        perf_plan_s* q = plans[b - 1];
+      const size_t rows_b = (size_t)h.halo_rows * W * sizeof(float);
+      if (h.up_rank >= 0) {
+        perf_plan_s* q = plans[h.up_rank];
         const float* theirs = power_buf ? q->band.pbuf : q->band.buf[which];
-        CK(cudaMemcpyAsync(mine, theirs + (size_t)q->H * W + (q->band.hb - hb) * W, hb * W * sizeof(float),
-                           cudaMemcpyDeviceToDevice, s));
+        CK(cudaMemcpyAsync(mine + (size_t)h.recv_up_row * W, theirs + (size_t)halo_plan(q, h.up_rank).send_down_row * W,
+                           rows_b, cudaMemcpyDeviceToDevice, xs));
       }
-      if (b < nb - 1) {  // bottom halo <- first hb rows of band b+1
-        perf_plan_s* q = plans[b + 1];
+      if (h.down_rank >= 0) {
+        perf_plan_s* q = plans[h.down_rank];
         const float* theirs = power_buf ? q->band.pbuf : q->band.buf[which];
-        CK(cudaMemcpyAsync(mine + (hb + h) * W, theirs + (size_t)q->band.hb * W, hb * W * sizeof(float),
-                           cudaMemcpyDeviceToDevice, s));
+        CK(cudaMemcpyAsync(mine + (size_t)h.recv_down_row * W, theirs + (size_t)halo_plan(q, h.down_rank).send_up_row * W,
+                           rows_b, cudaMemcpyDeviceToDevice, xs));
       }
     }
     return PERF_OK;
@@ -931,8 +1105,9 @@ perf_status perf_run_hotspot_bands_local(perf_plan_t* plans, int nb, const float
       const int steps = (int)std::min(tb, iters - i);
       for (int b = 0; b < nb; ++b) {
         Band& B = plans[b]->band;
-        if ((st = band_step(plans[b], B.buf[cur], B.buf[cur ^ 1], steps, s, B.peer_buf[0][cur ^ 1],
-                            B.peer_buf[1][cur ^ 1])) != PERF_OK)
+        perf_plan_s* p = plans[b];
+        if ((st = band_launch(p, B.buf[cur], B.buf[cur ^ 1], steps, (int)p->band_y0, (int)p->band_y0 + p->H, s,
+                              B.peer_buf[0][cur ^ 1], B.peer_buf[1][cur ^ 1])) != PERF_OK)
           return st;
       }
       if ((st = sync_all()) != PERF_OK) return st;
@@ -946,15 +1121,43 @@ perf_status perf_run_hotspot_bands_local(perf_plan_t* plans, int nb, const float
     }
     return PERF_OK;
   }
-  st = exchange(0, true);
-  if (st != PERF_OK) return st;
+  if ((st = exchange(0, true, s)) != PERF_OK) return st;
+  if ((st = exchange(0, false, s)) != PERF_OK) return st;
+  bool split = true;
+  for (int b = 0; b < nb; ++b) split = split && band_splits(plans[b]);
+  perf_plan_s* p0 = plans[0];
   int cur = 0;
   for (long long i = 0; i < iters; i += tb) {
-    if ((st = exchange(cur, false)) != PERF_OK) return st;
     const int steps = (int)std::min(tb, iters - i);
-    for (int b = 0; b < nb; ++b)
-      if ((st = band_step(plans[b], plans[b]->band.buf[cur], plans[b]->band.buf[cur ^ 1], steps, s)) != PERF_OK)
-        return st;
+    const bool last = i + tb >= iters;
+    if (split && !last) {  // every band's boundary rows, the exchange on p0's stream, every interior
+      for (int b = 0; b < nb; ++b) {
+        perf_plan_s* p = plans[b];
+        const int y0 = (int)p->band_y0, h = p->H, hb = p->band.hb;
+        if ((st = band_launch(p, p->band.buf[cur], p->band.buf[cur ^ 1], steps, y0, y0 + hb, s)) != PERF_OK) return st;
+        if ((st = band_launch(p, p->band.buf[cur], p->band.buf[cur ^ 1], steps, y0 + h - hb, y0 + h, s)) != PERF_OK)
+          return st;
+      }
+      CK(cudaEventRecord(p0->ev_b, s));
+      CK(cudaStreamWaitEvent(p0->s_x, p0->ev_b, 0));
+      if ((st = exchange(cur ^ 1, false, p0->s_x)) != PERF_OK) return st;
+      CK(cudaEventRecord(p0->ev_x, p0->s_x));
+      for (int b = 0; b < nb; ++b) {
+        perf_plan_s* p = plans[b];
+        const int y0 = (int)p->band_y0, h = p->H, hb = p->band.hb;
+        if ((st = band_launch(p, p->band.buf[cur], p->band.buf[cur ^ 1], steps, y0 + hb, y0 + h - hb, s)) != PERF_OK)
+          return st;
+      }
+      CK(cudaStreamWaitEvent(s, p0->ev_x, 0));
+    } else {
+      for (int b = 0; b < nb; ++b) {
+        perf_plan_s* p = plans[b];
+        if ((st = band_launch(p, p->band.buf[cur], p->band.buf[cur ^ 1], steps, (int)p->band_y0,
+                              (int)p->band_y0 + p->H, s)) != PERF_OK)
+          return st;
+      }
+      if (!last && (st = exchange(cur ^ 1, false, s)) != PERF_OK) return st;
+    }
     cur ^= 1;
   }
   for (int b = 0; b < nb; ++b) {
@@ -965,10 +1168,34 @@ perf_status perf_run_hotspot_bands_local(perf_plan_t* plans, int nb, const float
   return PERF_OK;
 }
 
-perf_status perf_error(perf_plan_t p, const void* exact, const void* approx, void* stream, double* err_out,
-                       long long* count_out) {
-  if (!p || !exact || !approx || !err_out) return fail(PERF_ERR_INVALID_ARG, "NULL argument");
+perf_status perf_run_hotspot_bands_local(perf_plan_t* plans, int nb, const float* temp_in, const float* power,
+                                         float* temp_out, void* stream) {
+  if (!plans || nb < 1 || !temp_in || !power || !temp_out) return fail(PERF_ERR_INVALID_ARG, "bad arguments");
   cudaStream_t s = static_cast<cudaStream_t>(stream);
+  const size_t W = plans[0]->W;
+  const long long iters = plans[0]->iters;
+  for (int b = 0; b < nb; ++b) {
+    perf_plan_s* p = plans[b];
+    if (!p || p->app != PERF_APP_HOTSPOT || (size_t)p->W != W || p->iters != iters || p->tblock != plans[0]->tblock)
+      return fail(PERF_ERR_INVALID_ARG, "band plans must be Hotspot plans of one grid (same ITERS, TBLOCK)");
+    if (p->tblock > 1 && p->rate.num > 0 && p->scheme != PERF_SCHEME_ROW && p->scheme != PERF_SCHEME_NONE)
+      return fail(PERF_ERR_UNSUPPORTED, "TBLOCK > 1 needs the NONE or ROW scheme");
+    if (b > 0 && p->band_y0 != plans[b - 1]->band_y0 + plans[b - 1]->H)
+      return fail(PERF_ERR_INVALID_ARG, "bands must be consecutive");
+    perf_status st = hotspot_prepare(p, true);
+    if (st != PERF_OK) return st;
+  }
+  auto enq = [&](cudaStream_t cs) { return bands_local_enqueue(plans, nb, temp_in, power, temp_out, cs); };
+  if (plans[0]->p2p) return enq(s);  // epoch counters live on the host
+  std::vector<const void*> key = {temp_in, power, temp_out};
+  for (int b = 0; b < nb; ++b) {  // (a perf_plan_set on any band plan changes its gen)
+    key.push_back(plans[b]);
+    key.push_back(reinterpret_cast<const void*>((uintptr_t)plans[b]->gen));
+  }
+  return graph_run(plans[0], key, s, enq);
+}
+
+static perf_status error_sums(perf_plan_s* p, const void* exact, const void* approx, cudaStream_t s, double h[3]) {
   if (!p->d_err) {
     if (cudaMalloc(&p->d_err, kp::error_scratch_doubles() * sizeof(double)) != cudaSuccess)
       return fail(PERF_ERR_OOM, "error scratch allocation");
@@ -976,13 +1203,85 @@ perf_status perf_error(perf_plan_t p, const void* exact, const void* approx, voi
   const long long n = (long long)p->batch * p->W * p->H;
   cudaError_t e = kp::launch_error(p->app == PERF_APP_MEDIAN, exact, approx, n, (int)p->metric, p->d_err, s);
   if (e != cudaSuccess) return cuda_fail(e, "perf_error launch");
-  double h[3];
-  CK(cudaMemcpyAsync(h, p->d_err + kp::error_scratch_doubles() - 3, sizeof h, cudaMemcpyDeviceToHost, s));
+  CK(cudaMemcpyAsync(h, p->d_err + kp::error_scratch_doubles() - 3, 3 * sizeof(double), cudaMemcpyDeviceToHost, s));
   CK(cudaStreamSynchronize(s));
+  return PERF_OK;
+}
+
+perf_status perf_error_finish(perf_plan_t p, const double h[3], double* err_out, long long* count_out) {
+  if (!p || !h || !err_out) return fail(PERF_ERR_INVALID_ARG, "NULL argument");
   const long long c = (long long)h[2];
   if (count_out) *count_out = c;
   if (p->metric == PERF_METRIC_ME) *err_out = h[1] > 0 ? h[0] / h[1] : 0.0;
   else *err_out = c > 0 ? h[0] / (double)c : 0.0;
+  return PERF_OK;
+}
+
+perf_status perf_error_sums(perf_plan_t p, const void* exact, const void* approx, void* stream, double sums[3]) {
+  if (!p || !exact || !approx || !sums) return fail(PERF_ERR_INVALID_ARG, "NULL argument");
+  return error_sums(p, exact, approx, static_cast<cudaStream_t>(stream), sums);
+}
+
+perf_status perf_error(perf_plan_t p, const void* exact, const void* approx, void* stream, double* err_out,
+                       long long* count_out) {
+  if (!p || !exact || !approx || !err_out) return fail(PERF_ERR_INVALID_ARG, "NULL argument");
+  double h[3];
+  perf_status st = error_sums(p, exact, approx, static_cast<cudaStream_t>(stream), h);
+  if (st != PERF_OK) return st;
+  return perf_error_finish(p, h, err_out, count_out);
+}
+
+perf_status perf_error_allreduce(perf_plan_t p, const void* exact, const void* approx, void* stream, double* err_out,
+                                 long long* count_out) {
+  if (!p || !exact || !approx || !err_out) return fail(PERF_ERR_INVALID_ARG, "NULL argument");
+  cudaStream_t s = static_cast<cudaStream_t>(stream);
+  double h[3];
+  perf_status st = error_sums(p, exact, approx, s, h);
+  if (st != PERF_OK) return st;
+  if (p->comm && p->nranks > 1) {  // (Σ terms, Σ|e|, count) summed over the ranks, in place on the device
+    double* d = p->d_err + kp::error_scratch_doubles() - 3;
+    ncclResult_t r = ncclAllReduce(d, d, 3, ncclFloat64, ncclSum, p->comm, s);
+    if (r != ncclSuccess) return fail(PERF_ERR_NCCL, std::string("error allreduce: ") + ncclGetErrorString(r));
+    CK(cudaMemcpyAsync(h, d, sizeof h, cudaMemcpyDeviceToHost, s));
+    CK(cudaStreamSynchronize(s));
+  }
+  return perf_error_finish(p, h, err_out, count_out);
+}
+
+perf_status perf_band_halo(perf_plan_t p, int rank, int nranks, perf_halo_plan* out) {
+  if (!p || !out) return fail(PERF_ERR_INVALID_ARG, "NULL argument");
+  if (nranks < 1 || rank < 0 || rank >= nranks) return fail(PERF_ERR_INVALID_ARG, "bad rank / nranks");
+  *out = halo_plan(p, rank);
+  const int Hg = p->global_h > 0 ? (int)p->global_h : p->H;
+  if ((p->band_y0 > 0 && rank == 0) || (p->band_y0 + p->H < Hg && rank == nranks - 1) ||
+      (p->band_y0 == 0 && rank > 0) || (p->band_y0 + p->H >= Hg && rank < nranks - 1))
+    return fail(PERF_ERR_INVALID_ARG, "band geometry (BAND_Y0, H, GLOBAL_H) does not match rank / nranks");
+  return PERF_OK;
+}
+
+perf_status perf_run_band(perf_plan_t p, void* in_band, void* out, void* stream) {
+  if (!p || !in_band || !out) return fail(PERF_ERR_INVALID_ARG, "NULL argument");
+  if (p->app == PERF_APP_HOTSPOT) return fail(PERF_ERR_UNSUPPORTED, "Hotspot bands run through perf_run_hotspot");
+  const int Hg = p->global_h > 0 ? (int)p->global_h : p->H, y0 = (int)p->band_y0, h = p->H;
+  if (y0 + h > Hg) return fail(PERF_ERR_INVALID_ARG, "band extends below GLOBAL_H");
+  if (p->scheme == PERF_SCHEME_STENCIL1 && y0 % (int)p->tile1_h != 0)
+    return fail(PERF_ERR_UNSUPPORTED, "STENCIL1 bands must start on a tile row (BAND_Y0 % TILE1_H == 0)");
+  cudaStream_t s = static_cast<cudaStream_t>(stream);
+  const perf_halo_plan hp = halo_plan(p, p->rank);
+  const int hb = hp.halo_rows;
+  const size_t es = elem_size(p->app), fin = (size_t)hp.buf_rows * p->W;
+  perf_status st = band_exchange_nccl(p, in_band, es, (int)p->batch, fin, s);
+  if (st != PERF_OK) return st;
+  KParams k;
+  unsigned grid;
+  size_t smem;
+  st = make_params(p, in_band, nullptr, out, (int)p->batch, y0 - hb, std::max(0, y0 - hb), std::min(Hg, y0 + h + hb), y0,
+                   y0, y0 + h, k, grid, smem);
+  if (st != PERF_OK) return st;
+  k.in_fstride = (long long)fin;
+  k.out_fstride = (long long)h * p->W;
+  cudaError_t e = dispatch(p, k, grid, smem, s);
+  if (e != cudaSuccess) return cuda_fail(e, "perf_run_band launch");
   return PERF_OK;
 }
 
@@ -1007,6 +1306,30 @@ perf_status perf_comm_init(perf_plan_t p, const void* uid, int rank, int nranks)
   p->comm = c;
   p->rank = rank;
   p->nranks = nranks;
+  // connect the ring neighbours now (a 4-byte exchange), not lazily inside the
+  // first (possibly graph-captured) halo exchange
+  if (nranks > 1) {
+    void* d = nullptr;
+    cudaStream_t ws = nullptr;
+    CK(cudaMalloc(&d, 16));
+    CK(cudaStreamCreateWithFlags(&ws, cudaStreamNonBlocking));
+    char* b = static_cast<char*>(d);
+    ncclGroupStart();
+    if (rank > 0) {
+      ncclSend(b, 4, ncclUint8, rank - 1, c, ws);
+      ncclRecv(b + 4, 4, ncclUint8, rank - 1, c, ws);
+    }
+    if (rank < nranks - 1) {
+      ncclSend(b + 8, 4, ncclUint8, rank + 1, c, ws);
+      ncclRecv(b + 12, 4, ncclUint8, rank + 1, c, ws);
+    }
+    ncclResult_t rr = ncclGroupEnd();
+    cudaError_t e = cudaStreamSynchronize(ws);
+    cudaStreamDestroy(ws);
+    cudaFree(d);
+    if (rr != ncclSuccess) return fail(PERF_ERR_NCCL, std::string("neighbour warm-up: ") + ncclGetErrorString(rr));
+    if (e != cudaSuccess) return cuda_fail(e, "neighbour warm-up");
+  }
   return PERF_OK;
 }
 
@@ -1077,6 +1400,11 @@ perf_status perf_destroy(perf_plan_t p) {
   if (p->d_stage_in) cudaFree(p->d_stage_in);
   if (p->d_stage_out) cudaFree(p->d_stage_out);
   host_pipe_free(p);
+  hotspot_graph_free(p);
+  if (p->s_cap) cudaStreamDestroy(p->s_cap);
+  if (p->s_x) cudaStreamDestroy(p->s_x);
+  if (p->ev_b) cudaEventDestroy(p->ev_b);
+  if (p->ev_x) cudaEventDestroy(p->ev_x);
   band_free(p);
   if (p->comm) ncclCommDestroy(p->comm);
   delete p;

@@ -62,7 +62,7 @@ def assert_close(app, r, got, want):
 @pytest.mark.parametrize("app,r", FLOAT_APPS)
 @pytest.mark.parametrize("scheme,rate,recon", VARIANTS)
 def test_float_apps_parity(app, r, scheme, rate, recon):
-    # 3 strips (last one ragged), 3 segments (last one ragged)
+    # 2 strips of 1024 columns (last one ragged), 3 segments (last one ragged)
     W, H = 1100, 300
     img = synth.image("natural", synth.SEED_C2 + 1, W, H)
     got = gpu_run(app, r, img, scheme, rate, recon)
@@ -162,16 +162,22 @@ def test_loaders_and_tiles_give_identical_bits():
                 assert np.array_equal(got, ref), (scheme, ld, th)
 
 
-@pytest.mark.parametrize("app,r", [("gaussian", 2), ("sobel", 1), ("gaussian", 1)])
-@pytest.mark.parametrize("den", [3, 4, 8])
+@pytest.mark.parametrize("app,r", [("gaussian", 2), ("sobel", 1), ("gaussian", 1), ("gauss_sobel", 2)])
+@pytest.mark.parametrize("den", [2, 3, 4, 8])
 @pytest.mark.parametrize("gbytes", [32, 128])
-def test_checker_keep_one_compact_slots(app, r, den, gbytes):
+@pytest.mark.parametrize("W", [2048, 512, 256])
+def test_checker_keep_one_compact_slots(app, r, den, gbytes, W):
     """Keep-one checkerboard with W a multiple of the warp width: every warp on
     the fast path, so the ring slots hold only the row's kept cells (kperf.cu
-    chk_compact).  == the oracle, and bit-identical to the scalar loader
-    (loader 3: full-width slots)."""
-    W, H = 2048, 300  # 2 strips, 3 segments (last ragged)
+    chk_compact; W 256 / 512: the 2-consumer-warp CTAs of narrow images).
+    == the oracle, and bit-identical to the scalar loader (loader 3:
+    full-width slots); the compact layout is asserted to be engaged."""
+    H = 300  # 3 segments (last ragged); W 2048: 2 strips
+    if W < 2048 and app == "gauss_sobel" and den == 8:
+        pytest.skip("covered at W 2048")
     img = synth.image("natural", 41 + den, W, H)
+    with kp.Plan(app, W, H, r, "checker", (den - 1, den), "li", granule_bytes=gbytes) as p:
+        assert p.get("chk_compact") == 1
     for recon in ("nn", "li"):
         got = gpu_run(app, r, img, "checker", (den - 1, den), recon, G_bytes=gbytes)
         want = oracle.run(oracle.params(app, W, H, r, "checker", (den - 1, den), recon, gbytes // 4), img)
@@ -327,9 +333,13 @@ def test_hotspot_parity(scheme, rate, recon, iters):
                                                ("row", (3, 4), "nn"), ("checker", (1, 2), "li")])
 @pytest.mark.parametrize("nb", [2, 3, 4])
 @pytest.mark.parametrize("tb", [1, 4])
-def test_hotspot_bands_equal_whole_grid(scheme, rate, recon, nb, tb):
+@pytest.mark.parametrize("overlap,graph", [(1, 1), (0, 0), (1, 0)])
+def test_hotspot_bands_equal_whole_grid(scheme, rate, recon, nb, tb, overlap, graph):
     """Sharding semantics: row bands with halo exchange == one grid, bit for bit
-    (tb > 1: temporally blocked launches, one halo exchange per launch)."""
+    (tb > 1: temporally blocked launches, one halo exchange per launch).
+    overlap: boundary rows first, their exchange on a second stream while the
+    interior computes; graph: the loop captured and replayed
+    (two calls: capture, then replay)."""
     if tb > 1 and scheme == "checker":
         pytest.skip("temporal blocking: NONE / ROW schemes")
     W, H, iters = 640, 200, 9
@@ -344,11 +354,13 @@ def test_hotspot_bands_equal_whole_grid(scheme, rate, recon, nb, tb):
     for b in range(nb):
         h = int(cuts[b + 1] - cuts[b])
         plans.append(kp.Plan("hotspot", W, h, 1, scheme, rate, recon, iters=iters, global_h=H,
-                             band_y0=int(cuts[b]), tblock=tb))
-    banded = torch.empty_like(Td)
-    kp.perf_run_hotspot_bands_local([q.handle for q in plans], Td, Pd, banded)
-    torch.cuda.synchronize()
-    assert torch.equal(banded, whole)
+                             band_y0=int(cuts[b]), tblock=tb, overlap=overlap, graph=graph))
+    for _ in range(2):
+        banded = torch.full_like(Td, float("nan"))
+        kp.perf_run_hotspot_bands_local([q.handle for q in plans], Td, Pd, banded)
+        torch.cuda.synchronize()
+        assert torch.equal(banded, whole)
+    assert plans[0].get("graph") == graph  # (2 would mean the capture failed)
     for q in plans:
         q.close()
 
