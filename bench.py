@@ -209,6 +209,20 @@ def max_over_ranks(ws, v):
     return float(t.item())
 
 
+def nccl_uid(kp, ws, rank):
+    """a libkperf NCCL unique id from rank 0, broadcast over the process group"""
+    import torch
+    import torch.distributed as dist
+    uid = kp.perf_comm_unique_id() if rank == 0 else bytes(128)
+    t = torch.tensor(list(uid), dtype=torch.uint8, device="cuda" if dist.get_backend() == "nccl" else "cpu")
+    dist.broadcast(t, 0)
+    return bytes(t.cpu().tolist())
+
+
+def min_over_ranks(ws, v):
+    return -max_over_ranks(ws, -v)
+
+
 def time_kernel(fn, stream, reps, warm):
     """average device time per call (ms), CUDA events on the launching stream"""
     import torch
@@ -365,7 +379,18 @@ def main():
         # exact kernel, same batch (speedup) and error at the stated MRE
         ms_exact = max_over_ranks(ws, time_kernel(lambda: exact.run(x, yex, stream), stream, args.steps,
                                                   args.warmup))
-        mre, cnt = plan.error(yex, y, stream)
+        if ws > 1:  # the error of the whole sharded batch: partial sums ncclAllReduce'd
+            uid = nccl_uid(kp, ws, rank)
+            try:
+                kp.perf_comm_init(plan.handle, uid, rank, ws)
+                mre, cnt = kp.perf_error_allreduce(plan.handle, yex, y, stream)
+            except kp.PerfError:  # (KPERF_BENCH_BACKEND=gloo test mode: ranks share a GPU, NCCL refuses)
+                import torch.distributed as dist
+                sums = torch.tensor(kp.perf_error_sums(plan.handle, yex, y, stream), dtype=torch.float64)
+                dist.all_reduce(sums)
+                mre, cnt = kp.perf_error_finish(plan.handle, sums.tolist())
+        else:
+            mre, cnt = plan.error(yex, y, stream)
         algo_b = bytes_per_px(app, cfg["scheme"], cfg["rate"]) * px_step
         achieved = algo_b / (ms * 1e-3) / 1e9
         kkey = f"{app}{cfg['r']}_{cfg['scheme']}_{cfg['rate'][0]}-{cfg['rate'][1]}_{cfg['recon']}"
@@ -393,7 +418,8 @@ def main():
             "speedup_vs_exact": ms_exact / ms, "exact_ms_per_step": ms_exact,
             "exact_mpixel_s": ws * px_step / (ms_exact * 1e-3) / 1e6,
             "error": {"metric": "mre" if app not in ("sobel", "gauss_sobel") else "me", "value": mre,
-                      "count": cnt},
+                      "count": cnt, "over": f"all {ws} ranks' frames (perf_error_allreduce)" if ws > 1
+                      else "the batch"},
             "hbm_gbs": achieved,
             "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
                          "frac": achieved / peak, "traffic": tr, "kernel": kkey,
@@ -412,6 +438,15 @@ def main():
             result["variants"] = bench_variants(kp, cfg, x, y, yex, stream, peak, ws)
         plan.close()
         exact.close()
+        if ws > 1 and args.config == "C2":  # the paths that really exchange data between GPUs
+            del x, y, yex
+            torch.cuda.empty_cache()
+            for key, fn in (("c4_row_bands", lambda: bench_c4_banded(kp, ws, rank, stream)),
+                            ("c2_row_bands", lambda: bench_c2_row_bands(kp, ws, rank, stream, args.steps))):
+                try:
+                    result[key] = fn()
+                except Exception as e:  # (e.g. NCCL refusing two ranks on one GPU under the gloo test mode)
+                    result[key] = {"error": f"{type(e).__name__}: {e}"}
     if rank == 0 and not args.no_cpu:
         result["cpu_baseline"] = cpu_baseline(cfg)
     if rank == 0:
@@ -490,6 +525,122 @@ def bench_variants(kp, cfg, x, y, yex, stream, peak, ws):
             p.close()
         ex.close()
     return out
+
+
+def hotspot_cone_ok(cfg, W, Hg, iters, x0, y0, w, h, got, scheme, rate, recon):
+    """oracle check of a w x h patch of a banded Hotspot result: the patch's
+    dependency cone (iters x (1 + den) rows / iters columns each side) is
+    generated on the device (synth, global rows), copied back and stepped by
+    oracle.hotspot_window; rows / columns at the window's edge are wrong only
+    outside the cone"""
+    import torch
+
+    import oracle
+    import synth
+    den = rate[1] if scheme in ("row", "checker") and rate[0] > 0 else 0
+    my, mx = iters * (1 + den), iters
+    wy0, wy1 = max(0, y0 - my), min(Hg, y0 + h + my)
+    wx0, wx1 = max(0, x0 - mx), min(W, x0 + w + mx)
+    T = torch.empty((wy1 - wy0, W), device="cuda")
+    P = torch.empty_like(T)
+    synth.hotspot_band_device(cfg["seed"], W, Hg, wy0, wy1 - wy0, T.data_ptr(), P.data_ptr())
+    torch.cuda.synchronize()
+    Tw = np.ascontiguousarray(T.cpu().numpy()[:, wx0:wx1].astype(np.float64))
+    Pw = np.ascontiguousarray(P.cpu().numpy()[:, wx0:wx1])
+    prm = oracle.params("hotspot", W, Hg, 1, scheme, rate, recon)
+    oracle.hotspot_window(prm, Tw, Pw, wx0, wy0, iters)
+    want = Tw[y0 - wy0:y0 - wy0 + h, x0 - wx0:x0 - wx0 + w]
+    return bool(np.all(np.abs(got.astype(np.float64) - want) <= 1e-5 * np.abs(want)))
+
+
+def bench_c4_banded(kp, ws, rank, stream, rows_per_gpu=2048, iters=20, reps=5):
+    """the C4 Hotspot as row bands over the N ranks, per-launch
+    NCCL halo exchange overlapped with the interior rows, the loop captured in
+    a CUDA graph.  16384 x (rows_per_gpu x N) cells, `iters` steps per call
+    (weak scaling).  Also timed with the exchange switched off
+    (PERF_KEY_EXCHANGE 0, results wrong at band edges) to give the halo's
+    share; each rank checks patches at both band edges against the oracle."""
+    import torch
+
+    import synth
+    cfg = CONFIGS["C4"]
+    W, Hg = cfg["W"], rows_per_gpu * ws
+    scheme, rate, recon = cfg["scheme"], cfg["rate"], cfg["recon"]
+    cuts = kp.band_cuts(Hg, ws)
+    y0, h = cuts[rank], cuts[rank + 1] - cuts[rank]
+    T = torch.empty((h, W), device="cuda")
+    P = torch.empty_like(T)
+    synth.hotspot_band_device(cfg["seed"], W, Hg, y0, h, T.data_ptr(), P.data_ptr(), stream.cuda_stream)
+    out = torch.empty_like(T)
+    uid = nccl_uid(kp, ws, rank)
+    res = {"grid": [W, Hg], "iters_per_call": iters, "bands": ws, "scheme": scheme, "rate": list(rate),
+           "recon": recon, "halo": "NCCL send/recv per launch, boundary rows first, exchange overlapped with the "
+                                   "interior rows, loop captured in a CUDA graph"}
+    times = {}
+    for xchg in (1, 0):
+        with kp.Plan("hotspot", W, h, 1, scheme, rate, recon, iters=iters, global_h=Hg, band_y0=y0,
+                     exchange=xchg) as p:
+            kp.perf_comm_init(p.handle, uid, rank, ws)
+            run = lambda: p.hotspot(T, P, out, stream)  # noqa: E731
+            barrier(ws)
+            times[xchg] = max_over_ranks(ws, time_kernel(run, stream, reps, 2))
+            if xchg:
+                res["graph"] = p.get("graph")
+                run()
+                torch.cuda.synchronize()
+                o = out.cpu().numpy()
+                ok = True
+                for x0, yy in ((1000, y0), (W - 4, y0 + h - 3), (8190, y0 + h // 2)):
+                    ok &= hotspot_cone_ok(cfg, W, Hg, iters, x0, yy, 4, 3, o[yy - y0:yy - y0 + 3, x0:x0 + 4],
+                                          scheme, rate, recon)
+                res["parity"] = "ok" if min_over_ranks(ws, 1.0 if ok else 0.0) > 0 else "MISMATCH"
+    cells = W * Hg * iters
+    res.update({"ms_per_call": times[1], "mcell_updates_s": cells / (times[1] * 1e-3) / 1e6,
+                "ms_per_call_no_exchange": times[0],
+                "halo_us_per_step": max(0.0, times[1] - times[0]) * 1e3 / iters,
+                "parity_check": "each rank: 4x3 patches at both band edges + the middle vs oracle.hotspot_window "
+                                "on the dependency cone"})
+    return res
+
+
+def bench_c2_row_bands(kp, ws, rank, stream, steps):
+    """one C2 batch (8 x 4096^2 fp32, Gaussian5 row 1/2 LI) split
+    into N row bands; every step perf_run_band fills the halo rows of all
+    frames with one NCCL group, then runs the band (strong scaling)"""
+    import torch
+
+    import synth
+    cfg = CONFIGS["C2"]
+    W, H, B = cfg["W"], cfg["H"], cfg["batch"]
+    cuts = kp.band_cuts(H, ws)
+    y0, h = cuts[rank], cuts[rank + 1] - cuts[rank]
+    uid = nccl_uid(kp, ws, rank)
+    with kp.Plan(cfg["app"], W, h, cfg["r"], cfg["scheme"], cfg["rate"], cfg["recon"], batch=B, global_h=H,
+                 band_y0=y0, granule_bytes=128) as p:
+        kp.perf_comm_init(p.handle, uid, rank, ws)
+        hp = kp.perf_band_halo(p.handle, rank, ws)
+        hb = hp["halo_rows"]
+        whole = torch.empty((B, H, W), device="cuda")
+        synth.image_device(cfg["cls"], cfg["seed"], W, H, B, whole.data_ptr(), False, stream.cuda_stream)
+        buf = torch.full((B, hp["buf_rows"], W), float("nan"), device="cuda")
+        buf[:, hb:hb + h] = whole[:, y0:y0 + h]  # own rows only; halos arrive by NCCL
+        del whole
+        out = torch.empty((B, h, W), device="cuda")
+        run = lambda: kp.perf_run_band(p.handle, buf, out, stream)  # noqa: E731
+        barrier(ws)
+        ms = max_over_ranks(ws, time_kernel(run, stream, steps, 3))
+        # sampled parity: rows at both band edges of frame 1 vs the oracle
+        import oracle
+        img = synth.image(cfg["cls"], cfg["seed"] + 1, W, H)
+        prm = oracle.params(cfg["app"], W, H, cfg["r"], cfg["scheme"], cfg["rate"], cfg["recon"])
+        ys = np.r_[y0, y0 + 1, y0 + h - 2, y0 + h - 1]
+        yy, xx = np.meshgrid(ys, np.arange(0, W, 11), indexing="ij")
+        want = oracle.run_pixels(prm, img, xx.ravel(), yy.ravel())
+        got = out[1].cpu().numpy()[yy.ravel() - y0, xx.ravel()]
+        ok = bool(np.all(np.abs(got - want) <= 1e-5 * np.abs(want)))
+    return {"workload": cfg["workload"] + f", one batch split into {ws} row bands", "ms_per_step": ms,
+            "mpixel_s": B * W * H / (ms * 1e-3) / 1e6, "scaling": "strong", "halo_rows": hb,
+            "parity": "ok" if min_over_ranks(ws, 1.0 if ok else 0.0) > 0 else "MISMATCH"}
 
 
 def bench_hotspot(args, cfg, ws, rank, local, stream, peak, peak_src):
