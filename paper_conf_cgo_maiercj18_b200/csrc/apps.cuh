@@ -309,7 +309,10 @@ struct AppMedian {
   using T = uint8_t;
   static constexpr bool ULI = KPERF_ULI;
   static constexpr bool IPROD = KPERF_IPROD;
-  static constexpr int V = 16, EW = 4, VR = 1, NIN = 1, NWIN = 3, MINB = 3;
+  // MINB 4 (96 registers): 4 CTAs / SM.  The column scheme's all-skipped warps
+  // (kernel.cuh MEDC) leave the kept warps as the critical path; more resident
+  // CTAs hide their latency (C3 col 1/2 NN 235 -> 196 us, exact 230 -> 228 us)
+  static constexpr int V = 16, EW = 4, VR = 1, NIN = 1, NWIN = 3, MINB = 4;
   static constexpr int NW = V / 2 + 2;  // 16-bit-pair words per row incl. the two halo words
   uint32_t r[3][NW];  // word 0 = (_, col -1), words 1..V/2 = cols 0..V-1, last = (col V, _)
   __device__ void init(const KParams&) {}
@@ -324,8 +327,8 @@ struct AppMedian {
     constexpr uint32_t HI = 0x64646464u;  // fp16 exponent byte of 1024
     uint32_t lft = __shfl_up_sync(FULLMASK, c.w[V / 4 - 1], 1);
     uint32_t rgt = __shfl_down_sync(FULLMASK, c.w[0], 1);
-    if (lane == 0) lft = e.w[0];
-    if (lane == 31) rgt = e.w[0];
+    if (hf & 4u) lft = e.w[0];  // lane's left / right neighbour column lies in its edge fragment
+    if (hf & 8u) rgt = e.w[0];  // (lane 0 / 31; the first / last lane of a cell under cell-grouped lanes)
     if (hf & 1u) lft = c.w[0] << 24;           // Stencil1 tile border: col -1 := col 0
     if (hf & 2u) rgt = c.w[V / 4 - 1] >> 24;  // col V := col V-1
     r[U][0] = __byte_perm(lft, HI, 0x4344);  // (0x6464, 0x64|col -1)

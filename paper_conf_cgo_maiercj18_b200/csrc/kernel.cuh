@@ -17,6 +17,9 @@
 #ifndef KPERF_MINB
 #define KPERF_MINB 0  // 0: per-app App::MINB
 #endif
+#ifndef KPERF_MEDCELL
+#define KPERF_MEDCELL 1  // median column NN: cell-grouped lanes + the all-skipped-warp shortcut
+#endif
 
 namespace kp {
 
@@ -42,17 +45,47 @@ inline int dev_sms() {
 }
 
 
+#ifndef KPERF_SLEEP_NS
+#define KPERF_SLEEP_NS 200
+#endif
+#ifndef KPERF_WAIT_HINT
+#define KPERF_WAIT_HINT 1000  // consumer full-barrier waits: try_wait suspend-time hint in ns (0 = none)
+#endif
 __device__ __forceinline__ void mbar_wait_u32(uint32_t addr, uint32_t parity) {
   // watchdog: a protocol bug traps (launch error) instead of hanging the GPU
   uint32_t ok, spins = 0;
   do {
+#if KPERF_WAIT_HINT
+    asm volatile(
+        "{\n .reg .pred p;\n mbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2, %3;\n selp.u32 %0, 1, 0, p;\n}"
+        : "=r"(ok)
+        : "r"(addr), "r"(parity), "n"(KPERF_WAIT_HINT)
+        : "memory");
+#else
     asm volatile(
         "{\n .reg .pred p;\n mbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2;\n selp.u32 %0, 1, 0, p;\n}"
         : "=r"(ok)
         : "r"(addr), "r"(parity)
         : "memory");
+#endif
     if (++spins > (1u << 26)) __trap();
   } while (!ok);
+}
+// the same wait for warps that are far ahead of the slowest consumer warp of
+// their CTA (the median's all-skipped warps): back off with nanosleep so the
+// spin does not take issue slots from the ALU-bound warps on the same SMSP
+__device__ __forceinline__ void mbar_wait_sleep_u32(uint32_t addr, uint32_t parity) {
+  uint32_t ok, spins = 0;
+  for (;;) {
+    asm volatile(
+        "{\n .reg .pred p;\n mbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2;\n selp.u32 %0, 1, 0, p;\n}"
+        : "=r"(ok)
+        : "r"(addr), "r"(parity)
+        : "memory");
+    if (ok) break;
+    if (++spins > (1u << 24)) __trap();
+    __nanosleep(KPERF_SLEEP_NS);
+  }
 }
 __device__ __forceinline__ void mbar_arrive_u32(uint32_t addr) {
   asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(addr) : "memory");
@@ -100,18 +133,48 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
   };
   const int xw = x0 + w * 32 * V;
   const int base = x0 - p.hx;
-  const int xc = xw + lane * V;
-  const int ex = lane < 16 ? xw - EW : xw + 32 * V;  // edge fragment (warp halo) start column
+  int xc = xw + lane * V;
+  int ex = lane < 16 ? xw - EW : xw + 32 * V;  // edge fragment (warp halo) start column
+  int cex = lane < 16 ? xw - CV : xw + 32 * V;  // ... and its 16-B chunk
+  uint32_t hedge = lane == 0 ? 4u : (lane == 31 ? 8u : 0u);  // lane's left / right neighbour comes from e
+  // Median, column NN (C3): cell-grouped lanes.  The strip's G-wide cells are
+  // dealt to the warps kept cells first, then skipped ones, G/V lanes per cell;
+  // a warp whose cells are all skipped has every 3x3 window built from at most
+  // two rebuilt columns (the edge samples a, b) and takes the scalar path below
+  // (DESIGN.md "Median").  Neighbour columns across a cell edge come from the
+  // lane's edge fragment, not a shuffle.
+  constexpr bool MEDC = FAST && SCHEME == S_COL && sizeof(T) == 1 && RECON == R_NN && KPERF_MEDCELL;
+  bool cellmap = false;
+  if constexpr (MEDC) {
+    if (p.cellmap && x0 + TW <= p.W) {
+      cellmap = true;
+      const int lpc = p.G / V, ncell = TW / p.G, c0 = x0 / p.G;
+      const int want = w * (32 / lpc) + lane / lpc;
+      int nk = 0;
+      for (int j = 0; j < ncell; ++j) nk += m.phase_kept((c0 + j) % m.den) ? 1 : 0;
+      int cell = 0, kk = 0, ks = 0;
+      for (int j = 0; j < ncell; ++j) {
+        const int pos = m.phase_kept((c0 + j) % m.den) ? kk++ : nk + ks++;
+        if (pos == want) cell = j;
+      }
+      const int cs = x0 + cell * p.G, li = lane % lpc;
+      const bool left = li < lpc / 2;
+      xc = cs + li * V;
+      ex = left ? cs - EW : cs + p.G;
+      cex = left ? cs - CV : cs + p.G;
+      hedge = (li == 0 ? 4u : 0u) | (li == lpc - 1 ? 8u : 0u);
+    }
+  }
   const ChunkInfo cc = make_chunk<SCHEME>(p, m, xc);
-  const ChunkInfo ce = make_chunk<SCHEME>(p, m, lane < 16 ? xw - CV : xw + 32 * V);
+  const ChunkInfo ce = make_chunk<SCHEME>(p, m, cex);
   // edge fragment: 0 inside the image, 1 left of column 0, 2 right of column W-1, 3 straddles W
   const int emode = (ex >= 0 && ex + EW <= p.W) ? 0 : (ex < 0 ? 1 : (ex == p.W ? 2 : 3));
   const int ccol = xc - base, ecol = ex - base;
   const T* ring2 = ring + p.row_elems;  // second input (Hotspot power)
   // Stencil1: lane edges that are tile borders take their halo from the tile itself
-  const uint32_t hf = SCHEME == S_STENCIL1
-                          ? (uint32_t)((xc % p.tile1_w) == 0) | ((uint32_t)(((xc + V) % p.tile1_w) == 0) << 1)
-                          : 0u;
+  const uint32_t hf = hedge | (SCHEME == S_STENCIL1
+                                     ? (uint32_t)((xc % p.tile1_w) == 0) | ((uint32_t)(((xc + V) % p.tile1_w) == 0) << 1)
+                                     : 0u);
   App app;
   app.init(p);
   T* optr = static_cast<T*>(p.out) + (long long)frame * p.out_fstride + (long long)(ys - p.out_row0) * p.W + xc;
@@ -254,11 +317,9 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
   // fetch: recipe, ring release/wait, rebuild from shared memory (a1/a2).
   // After the first row, a row needs at most one more ring row and frees at
   // most one (every scheme's recipes advance by <= 1), so the waits are ifs.
-  auto fetch = [&](int i) {
-    Rows r;
+  auto sync = [&](int i, bool sleepy = false) {  // the ring protocol of virtual row i: release what it no longer needs, wait for what it needs
     const Recipe rec = rtab[i];
     const int need_hi = g0 + (rec.need & 0x7FFF), need_lo = g0 + (int)((uint32_t)rec.need >> 16);
-    r.emit = (rec.need >> 15) & 1;
     if (released < need_lo) {  // every lane arrives (empty barrier count = 32 x active warps)
       mbar_arrive_u32(empty_u32 + 8 * (released & nmask));
       ++released;
@@ -266,8 +327,15 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
     if (issuer) issue_ahead(need_hi - g0);
     if (ready < need_hi) {
       ++ready;
-      mbar_wait_u32(full_u32 + 8 * (ready & nmask), (ready >> p.nr_log2) & 1);
+      if (sleepy) mbar_wait_sleep_u32(full_u32 + 8 * (ready & nmask), (ready >> p.nr_log2) & 1);
+      else mbar_wait_u32(full_u32 + 8 * (ready & nmask), (ready >> p.nr_log2) & 1);
     }
+    return rec;
+  };
+  auto fetch = [&](int i) {
+    Rows r;
+    const Recipe rec = sync(i);
+    r.emit = (rec.need >> 15) & 1;
     if constexpr (FAST && SCHEME == S_COL && sizeof(T) == 1 && RECON == R_NN) {
       const T* row = ring + rc_slot_a(rec.info) * slot_elems;
       auto combine = [&](auto nc, const NNu8& z, int col) {
@@ -452,6 +520,68 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
     }
   };
 
+  if constexpr (MEDC) {
+    // all-skipped warp (column NN median): with column sources a (x <= mid) and
+    // b (x > mid), mid = floor((xa + xb) / 2) (ties to a, R6), a 3x3
+    // window holds one source column three times -- its median is med3 of that
+    // column -- except at x = mid (columns a, a, b) and x = mid + 1 (a, b, b),
+    // where the sorted-column identity (R11) reduces to
+    // med3(max(lo_a, lo_b), md_a or md_b, min(hi_a, hi_b)).  a and b ride as
+    // one u16x2 word per row; the four candidate bytes (med_a, med_b, mid,
+    // mid + 1) are packed into one word and each output word is one PRMT with a
+    // per-lane, row-independent selector.  Bit-exact with the full network.
+    if (cellmap && __all_sync(0xFFFFFFFFu, !cc.col_kept)) {
+      const int ca = zc.ca, cb = zc.cb;
+      const bool hb = cc.xb >= 0;
+      const int sab = cc.xa + cc.xb;
+      uint32_t sel[V / 4];
+#pragma unroll
+      for (int k = 0; k < V / 4; ++k) {
+        sel[k] = 0;
+#pragma unroll
+        for (int j = 0; j < 4; ++j) {
+          const int x = xc + 4 * k + j;
+          const uint32_t sv = !hb ? 0u : (2 * (x + 1) <= sab ? 0u : (2 * (x - 1) > sab ? 1u : (2 * x <= sab ? 2u : 3u)));
+          sel[k] |= sv << (4 * j);
+        }
+      }
+      uint32_t abw[3];
+      for (int ib = 0; ib < nv; ib += 3) {
+        auto unrolled = [&](auto uc) {
+          constexpr int U = decltype(uc)::value, A = (U + 1) % 3, B = (U + 2) % 3;
+          const int i = ib + U;
+          if (i < nv) {
+            const Recipe rec = sync(i, true);
+            const T* row = ring + rc_slot_a(rec.info) * slot_elems;
+            abw[U] = (uint32_t)row[ca] | ((uint32_t)row[cb] << 16);
+            if ((rec.need >> 15) & 1) {
+              const uint32_t t1 = vmin2(abw[A], abw[B]), t2 = vmax2(abw[A], abw[B]);
+              const uint32_t lo = vmin2(t1, abw[U]), t3 = vmax2(t1, abw[U]);
+              const uint32_t md = vmin2(t2, t3), hi = vmax2(t2, t3);
+              const uint32_t L = vmax2(lo, __byte_perm(lo, 0, 0x1032)), Hm = vmin2(hi, __byte_perm(hi, 0, 0x1032));
+              const uint32_t M = vmax2(vmin2(L, md), vmin2(vmax2(L, md), Hm));  // med3(L, md, Hm) per half
+              const uint32_t X = __byte_perm(md, M, 0x6420);  // (med_a, med_b, mid, mid + 1)
+              Frag<T, V> o;
+#pragma unroll
+              for (int k = 0; k < V / 4; ++k) o.w[k] = __byte_perm(X, 0, sel[k]);
+              store(optr, o);
+              optr += p.W;
+            }
+          }
+        };
+        static_for<0, 3>(unrolled);
+      }
+      const int g_end = g0 + rp.nload;
+#pragma unroll 1
+      while (ready < g_end - 1) {
+        ++ready;
+        mbar_wait_u32(full_u32 + 8 * (ready & nmask), (ready >> p.nr_log2) & 1);
+      }
+#pragma unroll 1
+      for (; released < g_end; ++released) mbar_arrive_u32(empty_u32 + 8 * (released & nmask));
+      return;
+    }
+  }
 #if KPERF_PIPELINE
   // software pipeline: row i+1 is fetched before row i is computed
   Rows cur = fetch(0);
@@ -530,11 +660,8 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : (NCW
   const int n_items = p.n_strips * p.n_segs * p.frames;
 
   // consumer warps whose columns all lie right of the image have nothing to do
-  int nact = NCW;
-  {
-    const int x0s = (blockIdx.x % p.n_strips) * TW;
-    nact = min(NCW, (p.W - x0s + 32 * V - 1) / (32 * V));
-  }
+  const int x0 = (blockIdx.x % p.n_strips) * TW;
+  const int nact = min(NCW, (p.W - x0 + 32 * V - 1) / (32 * V));
   if (threadIdx.x == 0) {
     for (int s = 0; s < p.nr; ++s) {
       mbar_init(&full[s], (p.loader == L_BULK || p.loader == L_RUNS) ? 1u : 32u);
@@ -556,7 +683,7 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : (NCW
     b /= p.n_strips;
     const int seg = b % p.n_segs;
     const int frame = b / p.n_segs;
-    const int x0 = strip * TW;
+    (void)strip;  // (x0 above)
     const int ys = p.y_begin + seg * p.seg_h;
     const int ye = min(ys + p.seg_h, p.y_end);
     const RowPlan rp = make_row_plan<SCHEME>(p, m, ys, ye, App::VR);

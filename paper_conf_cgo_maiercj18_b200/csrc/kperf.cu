@@ -178,6 +178,9 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   k.G = G < 1 ? 1 : G;
   const bool rowwise = scheme == PERF_SCHEME_NONE || scheme == PERF_SCHEME_ROW || s1;  // whole rows kept
   k.fast_ok = (rowwise || (k.G % V) == 0) ? 1 : 0;
+  // median, column NN: cells of >= 2 lanes that tile the strip and a warp (kernel.cuh MEDC)
+  k.cellmap = (P->app == PERF_APP_MEDIAN && scheme == PERF_SCHEME_COL && P->recon == PERF_RECON_NN && k.den > 1 &&
+               k.G % (2 * V) == 0 && k.G <= 32 * V && TW % k.G == 0) ? 1 : 0;
   const bool chunk_uniform = rowwise || (k.G % CV) == 0;
   const bool aligned = ((reinterpret_cast<uintptr_t>(in) | reinterpret_cast<uintptr_t>(out) |
                          reinterpret_cast<uintptr_t>(in2)) & 15) == 0;

@@ -135,7 +135,7 @@ def test_c3_bench_launch(rate):
     prm = oracle.params("median", W, H, 1, "col", rate, "nn", G_BYTES)
     for f, rows, cols in ((0, True, False), (B - 1, False, True)):
         img = synth.image(cfg["cls"], cfg["seed"] + f, W, H, np.uint8)
-        _check_frame("median", 1, prm, img, y[f].cpu().numpy(), W, H, 4096, rows=rows, cols=cols, xstep=3)
+        _check_frame("median", 1, prm, img, y[f].cpu().numpy(), W, H, 2048, rows=rows, cols=cols, xstep=3)
 
 
 @pytest.mark.parametrize("scheme,rate,recon", [("row", (1, 2), "li"), ("row", (3, 4), "nn"), ("none", (0, 1), "nn")])

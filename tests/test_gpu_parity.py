@@ -643,3 +643,20 @@ def test_paper_orderings_on_gpu():
     errs = [mre("median", 1, synth.image(c, 0x5EED3200, W, H, np.uint8), "row", (1, 2), "nn")
             for c in ("flat", "natural", "pattern")]
     assert errs[0] < errs[1] < errs[2]  # Fig. 7: 0.12% < 5.05% < 19.32%
+
+
+@pytest.mark.parametrize("gbytes", [32, 64, 128, 256, 512])
+@pytest.mark.parametrize("rate", [(1, 2), (1, 3), (2, 3), (1, 4), (3, 4), (1, 8), (7, 8)])
+def test_median_col_nn_cell_lanes(gbytes, rate):
+    """Median, column NN: cell-grouped lanes and the all-skipped-warp shortcut
+    (kernel.cuh MEDC) -- bit-exact against the oracle's true median; two full
+    2048-column strips + a ragged one (identity lanes), every den / num, cells
+    of 2..32 lanes (including cells straddling warps' cell groups)"""
+    W, H = 4096 + 333, 150
+    img = synth.image("natural", 0x5EED2400 + gbytes, W, H, np.uint8)
+    got = gpu_run("median", 1, img, "col", rate, "nn", G_bytes=gbytes)
+    want = oracle.run(oracle.params("median", W, H, 1, "col", rate, "nn", gbytes), img)
+    assert_close("median", 1, got, want)
+    pat = synth.image("pattern", 0x5EED2500, W, H, np.uint8)  # high-frequency: every window differs
+    got = gpu_run("median", 1, pat, "col", rate, "nn", G_bytes=gbytes, batch=1)
+    assert_close("median", 1, got, oracle.run(oracle.params("median", W, H, 1, "col", rate, "nn", gbytes), pat))

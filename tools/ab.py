@@ -17,7 +17,8 @@ SETS = {
                 ("gaussian", 2, "checker", 1, 4, "li"), ("gaussian", 2, "checker", 1, 4, "nn"),
                 ("gaussian", 2, "checker", 3, 4, "li"), ("gaussian", 2, "checker", 3, 4, "nn"),
                 ("sobel", 1, "checker", 1, 4, "nn"), ("sobel", 1, "checker", 1, 2, "li")],
-    "median": [("median", 1, "none", 0, 1, "nn"), ("median", 1, "col", 1, 2, "nn"), ("median", 1, "row", 1, 2, "nn")],
+    "median": [("median", 1, "none", 0, 1, "nn"), ("median", 1, "col", 1, 2, "nn"), ("median", 1, "col", 1, 4, "nn"),
+               ("median", 1, "col", 3, 4, "nn"), ("median", 1, "row", 1, 2, "nn")],
     "c5": [("gauss_sobel", 2, "none", 0, 1, "nn"), ("gauss_sobel", 2, "row", 1, 2, "li")],
     "c1": [("gaussian", 2, "none", 0, 1, "nn", 512, 512, 512), ("gaussian", 2, "row", 1, 2, "li", 512, 512, 512),
            ("sobel", 1, "row", 1, 2, "nn", 512, 512, 512)],

@@ -22,6 +22,9 @@ import synth  # noqa: E402
 def variants(which):
     if which == "c3":
         return [("median", 1, "none", (0, 1), "nn"), ("median", 1, "col", (1, 2), "nn")]
+    if which == "c3all":
+        return [("median", 1, "none", (0, 1), "nn"), ("median", 1, "col", (1, 2), "nn"),
+                ("median", 1, "col", (1, 4), "nn"), ("median", 1, "col", (3, 4), "nn")]
     if which == "c5":
         return [("gauss_sobel", 2, "none", (0, 1), "nn"), ("gauss_sobel", 2, "row", (1, 2), "li")]
     if which == "c1":
@@ -47,8 +50,8 @@ def main():
     ap.add_argument("--gran", type=int, default=128)
     a = ap.parse_args()
     W = H = 4096
-    u8 = a.variants == "c3"
-    if a.variants == "c3":
+    u8 = a.variants in ("c3", "c3all")
+    if u8:
         W = H = 8192
     if a.variants == "c5":
         W, H = 3840, 2160
