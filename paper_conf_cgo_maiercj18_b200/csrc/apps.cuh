@@ -61,6 +61,25 @@ __device__ __forceinline__ float deriv(const float* x) {
   return fmaf(2.f, x[3] - x[1], x[4] - x[0]);
 }
 
+// the same passes on the output column pair (2j, 2j+1), x = &x[2j]: per column
+// the operations and their order are those of smooth / deriv (bit-identical),
+// issued as paired fp32 ops (FADD2 / FFMA2) where both operands sit in aligned
+// register pairs -- x[2j] is aligned when R = 2 (x[R + i] = c.v[i]), x[2j + 1]
+// when R = 1 -- and as scalar ops otherwise.  Gaussian5: 5 instructions per
+// column pair instead of 8.
+template <int R>
+__device__ __forceinline__ f2 smooth_pair(const float* x) {
+  if (R == 1) return fma2(splat2(2.f), pk2(x[1], x[2]), pk2(x[0] + x[2], x[1] + x[3]));
+  const f2 a = add2(pk2(x[0], x[1]), pk2(x[4], x[5]));
+  const f2 b = pk2(x[1] + x[3], x[2] + x[4]);
+  return fma2(splat2(6.f), pk2(x[2], x[3]), fma2(splat2(4.f), b, a));
+}
+template <int R>
+__device__ __forceinline__ f2 deriv_pair(const float* x) {
+  if (R == 1) return pk2(x[2] - x[0], x[3] - x[1]);
+  return fma2(splat2(2.f), pk2(x[3] - x[1], x[4] - x[2]), sub2(pk2(x[4], x[5]), pk2(x[0], x[1])));
+}
+
 // ---------------------------------------------------------------------------
 template <int R>
 struct AppGauss {  // K1 Gaussian, binomial (2R+1)^2, fp32
@@ -76,7 +95,7 @@ struct AppGauss {  // K1 Gaussian, binomial (2R+1)^2, fp32
     float x[V + 2 * R];
     ext_row<R, EW, V>(c, e, lane, hf, x);
 #pragma unroll
-    for (int j = 0; j < V / 2; ++j) h[U][j] = pk2(smooth<R>(x + 2 * j), smooth<R>(x + 2 * j + 1));
+    for (int j = 0; j < V / 2; ++j) h[U][j] = smooth_pair<R>(x + 2 * j);
     const f2 scale = splat2(R == 1 ? 1.f / 16.f : 1.f / 256.f);
     Frag<float, V> o;
 #pragma unroll
@@ -108,8 +127,8 @@ struct AppSobel {  // K5 Sobel, |(Gx, Gy)|, fp32
     ext_row<R, EW, V>(c, e, lane, hf, x);
 #pragma unroll
     for (int j = 0; j < V / 2; ++j) {
-      sx[U][j] = pk2(smooth<R>(x + 2 * j), smooth<R>(x + 2 * j + 1));
-      dx[U][j] = pk2(deriv<R>(x + 2 * j), deriv<R>(x + 2 * j + 1));
+      sx[U][j] = smooth_pair<R>(x + 2 * j);
+      dx[U][j] = deriv_pair<R>(x + 2 * j);
     }
     Frag<float, V> o;
 #pragma unroll
@@ -222,7 +241,7 @@ struct AppGaussSobel {
     float x[V + 4];  // columns xc-2 .. xc+V+1
     ext_row<2, EW, V>(c, e, lane, 0u, x);
 #pragma unroll
-    for (int j = 0; j < V / 2; ++j) hh[H4][j] = pk2(smooth<2>(x + 2 * j), smooth<2>(x + 2 * j + 1));
+    for (int j = 0; j < V / 2; ++j) hh[H4][j] = smooth_pair<2>(x + 2 * j);
     {  // edge column (lane 0: xc-1 from e = cols xc-4..xc-1; lane 31: xc+V from e = cols xc+V..xc+V+3)
       float t[5];
       if (lane < 16) { t[0] = e.v[1]; t[1] = e.v[2]; t[2] = e.v[3]; t[3] = c.v[0]; t[4] = c.v[1]; }

@@ -448,8 +448,14 @@ __device__ __forceinline__ Frag<T, N> ldf(const T* p) {
   constexpr int B = N * (int)sizeof(T);
   static_assert(B == 4 || B == 8 || B == 16 || B == 32, "fragment size");
   if constexpr (B == 32) {
+#ifdef KPERF_PROBE_NOCONFLICT  // experiment (wrong results): the same loads at a 16-B lane stride
+    const T* q = p - (threadIdx.x & 31) * (16 / sizeof(T));
+    reinterpret_cast<uint4*>(&f)[0] = reinterpret_cast<const uint4*>(q)[0];
+    reinterpret_cast<uint4*>(&f)[1] = reinterpret_cast<const uint4*>(q)[32];
+#else
     reinterpret_cast<uint4*>(&f)[0] = reinterpret_cast<const uint4*>(p)[0];
     reinterpret_cast<uint4*>(&f)[1] = reinterpret_cast<const uint4*>(p)[1];
+#endif
   } else if constexpr (B == 16) *reinterpret_cast<uint4*>(&f) = *reinterpret_cast<const uint4*>(p);
   else if constexpr (B == 8) *reinterpret_cast<uint2*>(&f) = *reinterpret_cast<const uint2*>(p);
   else *reinterpret_cast<uint32_t*>(&f) = *reinterpret_cast<const uint32_t*>(p);

@@ -35,10 +35,18 @@ __device__ __forceinline__ bool mbar_try_wait(uint64_t* bar, uint32_t parity) {
   return ok != 0;
 }
 
+#ifndef KPERF_PROD_SLEEP
+#define KPERF_PROD_SLEEP 0  // producer empty-slot wait: nanosleep back-off between polls (ns, 0 = spin)
+#endif
+// (the producer waits for ring slots to be released; a spinning producer warp
+// takes issue slots from the consumer warp that shares its SM sub-partition)
 __device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t parity) {
   uint32_t spins = 0;
   while (!mbar_try_wait(bar, parity)) {
     if (++spins > (1u << 26)) __trap();  // watchdog: trap instead of hanging
+#if KPERF_PROD_SLEEP
+    __nanosleep(KPERF_PROD_SLEEP);
+#endif
   }
 }
 

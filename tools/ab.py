@@ -23,6 +23,8 @@ SETS = {
     "c1": [("gaussian", 2, "none", 0, 1, "nn", 512, 512, 512), ("gaussian", 2, "row", 1, 2, "li", 512, 512, 512),
            ("sobel", 1, "row", 1, 2, "nn", 512, 512, 512)],
 }
+SETS["row34"] = [("gaussian", 2, "row", 3, 4, "nn"), ("gaussian", 2, "row", 3, 4, "li"), ("sobel", 1, "row", 3, 4, "nn"),
+                 ("sobel", 1, "row", 3, 4, "li"), ("gaussian", 2, "none", 0, 1, "nn"), ("sobel", 1, "none", 0, 1, "nn")]
 SETS["all"] = SETS["row"] + SETS["col"] + SETS["checker"]
 
 CHILD = r'''
