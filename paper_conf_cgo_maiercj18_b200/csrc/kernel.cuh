@@ -488,7 +488,7 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
       return;
     }
 #endif
-    if (FAST && KPERF_ST256 && V * sizeof(T) == 32 && p.vec32) {  // xc % V == 0, W % 8 == 0, 32-B base
+    if (FAST && KPERF_ST256 && V * sizeof(T) == 32) {  // (the fast path of 32-B lane chunks requires p.vec32)
       st_global_v8(dst, reinterpret_cast<const uint4*>(&o)[0], reinterpret_cast<const uint4*>(&o)[1]);
     } else if (FAST) {
 #pragma unroll
@@ -703,7 +703,10 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : (NCW
       // either inside or starting exactly at W (then it is the clamped border)
       const int exr = xw + 32 * V;
       const bool edges_ok = (exr + App::EW <= p.W) || (exr == p.W);
-      if (p.fast_ok && p.vec_io && xw + 32 * V <= p.W && edges_ok)
+      // (32-B lane chunks: the fast path stores them with one 256-bit store, so
+      // it also needs p.vec32 -- 32-B aligned output chunks; else generic)
+      const bool st_ok = !(KPERF_ST256 && V * sizeof(T) == 32) || p.vec32;
+      if (p.fast_ok && p.vec_io && st_ok && xw + 32 * V <= p.W && edges_ok)
         consumer_fast<App, SCHEME, RECON, NCW>(p, m, rp, x0, frame, ys, ye, g0, full_u32, empty_u32, ring,
                                                slot_elems, rtab, ctab);
       else
