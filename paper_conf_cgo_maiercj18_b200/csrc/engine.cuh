@@ -511,12 +511,22 @@ __device__ __forceinline__ uint8_t li_px(uint8_t a, uint8_t b, int da, int db) {
 //   info  slot_a | slot_b << 8 | ym << 16 | da << 20 | db << 24 | kept << 28 |
 //         li << 29 | has_a << 30 | has_b << 31
 //   wa    LI weight of the lower sample: value = b + (a - b) * wa, wa = db/(da+db)
+//   oa, ob  byte offsets of slot_a / slot_b in the ring (the fast paths add them
+//         to a per-lane column address: one IADD per source row, no slot index math)
 // Row scheme: a kept row, and an NN-rebuilt row, are plain copies of slot_a.
-struct Recipe {
-  int y, need;
-  uint32_t info;
+// 32 B: the first half {oa, ob, need, wa} is what the row scheme's fast path
+// reads -- one LDS.128 per row.
+struct __align__(16) Recipe {
+  int oa, ob, need;
   float wa;
+  int y;
+  uint32_t info;
+  int pad0, pad1;
 };
+template <typename T>
+__device__ __forceinline__ const T* ring_at(const T* ring, int off) {
+  return reinterpret_cast<const T*>(reinterpret_cast<const char*>(ring) + off);
+}
 
 __device__ __forceinline__ int rc_slot_a(uint32_t i) { return (int)(i & 0xFF); }
 __device__ __forceinline__ int rc_slot_b(uint32_t i) { return (int)((i >> 8) & 0xFF); }
@@ -552,7 +562,8 @@ __device__ __forceinline__ int virtual_row(const KParams& p, const RowPlan& rp, 
 }
 
 template <int SCHEME, int RECON>
-__device__ __forceinline__ Recipe make_recipe(const KParams& p, const Mask& m, const RowPlan& rp, int y, int emit) {
+__device__ __forceinline__ Recipe make_recipe(const KParams& p, const Mask& m, const RowPlan& rp, int y, int emit,
+                                              int slot_bytes) {
   Recipe r;
   const int ym = y % m.den, nmask = p.nr - 1;
   int need_hi, need_lo, sa = 0, sb = 0, da = 1, db = 1, kept = 1, li = 0, ha = 0, hb = 0;
@@ -597,6 +608,9 @@ __device__ __forceinline__ Recipe make_recipe(const KParams& p, const Mask& m, c
            ((uint32_t)db << 24) | ((uint32_t)kept << 28) | ((uint32_t)li << 29) | ((uint32_t)ha << 30) |
            ((uint32_t)hb << 31);
   r.wa = wa;
+  r.oa = sa * slot_bytes;
+  r.ob = sb * slot_bytes;
+  r.pad0 = r.pad1 = 0;
   return r;
 }
 
@@ -683,16 +697,17 @@ __device__ __forceinline__ Frag<T, N> rebuild_frag(const KParams& p, const Mask&
                                                    const Recipe& rec, const ChunkInfo& ci, const T* ring,
                                                    int slot_elems, int col, int fx, int base) {
   const uint32_t info = rec.info;
-  if (SCHEME == S_NONE || SCHEME == S_STENCIL1) return ldf<T, N>(ring + rc_slot_a(info) * slot_elems + col);
+  if (SCHEME == S_NONE || SCHEME == S_STENCIL1) return ldf<T, N>(ring_at(ring, rec.oa) + col);
   if constexpr (SCHEME == S_ROW && ULI && RECON == R_LI && sizeof(T) == 4) {
-    const Frag<T, N> a = ldf<T, N>(ring + rc_slot_a(info) * slot_elems + col);
-    const Frag<T, N> b = ldf<T, N>(ring + rc_slot_b(info) * slot_elems + col);
+    const Frag<T, N> a = ldf<T, N>(ring_at(ring, rec.oa) + col);
+    const Frag<T, N> b = ldf<T, N>(ring_at(ring, rec.ob) + col);
     return lerp_frag<N>(a, b, rec.wa);
   }
   if (SCHEME == S_ROW) {
-    if (RECON == R_NN || rc_kept(info)) return ldf<T, N>(ring + rc_slot_a(info) * slot_elems + col);
-    const Frag<T, N> a = ldf<T, N>(ring + rc_slot_a(info) * slot_elems + col);
-    const Frag<T, N> b = ldf<T, N>(ring + rc_slot_b(info) * slot_elems + col);
+    if (RECON == R_NN) return ldf<T, N>(ring_at(ring, rec.oa) + col);
+    const Frag<T, N> a = ldf<T, N>(ring_at(ring, rec.oa) + col);
+    if (rec.oa == rec.ob) return a;  // kept (or NN-rebuilt) row: one source
+    const Frag<T, N> b = ldf<T, N>(ring_at(ring, rec.ob) + col);
     if constexpr (sizeof(T) == 4) return lerp_frag<N>(a, b, rec.wa);
     else return li_frag<N>(a, b, rc_da(info), rc_db(info));
   }

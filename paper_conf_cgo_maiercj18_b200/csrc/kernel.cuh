@@ -337,7 +337,7 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
     const Recipe rec = sync(i);
     r.emit = (rec.need >> 15) & 1;
     if constexpr (FAST && SCHEME == S_COL && sizeof(T) == 1 && RECON == R_NN) {
-      const T* row = ring + rc_slot_a(rec.info) * slot_elems;
+      const T* row = ring_at(ring, rec.oa);
       auto combine = [&](auto nc, const NNu8& z, int col) {
         constexpr int N = decltype(nc)::value;
         Frag<T, N> f = ldf<T, N>(row + col);
@@ -411,7 +411,7 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
       r.e = emode == 0 ? el : eb;
       if constexpr (App::NIN > 1) r.c2 = rebuild_frag<T, V, SCHEME, RECON>(p, m, rp, rec, cc, ring2, slot_elems, ccol, xc, base);
     } else if constexpr (COLF) {
-      const float* row = reinterpret_cast<const float*>(ring) + rc_slot_a(rec.info) * slot_elems;
+      const float* row = reinterpret_cast<const float*>(ring_at(ring, rec.oa));
       auto colrow = [&](auto nc, const ColF& z, int col, const float4* wt) {
         constexpr int N = decltype(nc)::value;
         const Frag<float, N> c = ldf<float, N>(row + col);
@@ -552,7 +552,7 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
           const int i = ib + U;
           if (i < nv) {
             const Recipe rec = sync(i, true);
-            const T* row = ring + rc_slot_a(rec.info) * slot_elems;
+            const T* row = ring_at(ring, rec.oa);
             abw[U] = (uint32_t)row[ca] | ((uint32_t)row[cb] << 16);
             if ((rec.need >> 15) & 1) {
               const uint32_t t1 = vmin2(abw[A], abw[B]), t2 = vmax2(abw[A], abw[B]);
@@ -695,7 +695,7 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : (NCW
       for (int i = lane; i < nv; i += 32) {
         int emit;
         const int y = virtual_row<SCHEME>(p, rp, ys, ye, App::VR, i, emit);
-        rtab[i] = make_recipe<SCHEME, RECON>(p, m, rp, y, emit);
+        rtab[i] = make_recipe<SCHEME, RECON>(p, m, rp, y, emit, slot_elems * (int)sizeof(T));
       }
       __syncwarp();
       const int xw = x0 + (warp - cw0) * 32 * V;
