@@ -75,15 +75,21 @@ def load_peaks():
     return 6650.0, "fallback (B200_PROFILING.md)"
 
 
-def ncu_traffic(kernel_key):
-    """per-launch DRAM bytes from a committed ncu --set full capture, if present"""
+def ncu_entry(config, kernel_key):
+    """per-launch ncu counters of this config's kernel in bench's launch
+    configuration (profiles/ncu_traffic.json, written by tools/ncu_traffic.py)"""
     p = os.path.join(ROOT, "profiles", "ncu_traffic.json")
     if not os.path.exists(p):
         return None
     try:
-        return json.load(open(p)).get(kernel_key)
+        return json.load(open(p)).get(f"{config}/{kernel_key}")
     except Exception:
         return None
+
+
+def ncu_traffic(config, kernel_key):
+    e = ncu_entry(config, kernel_key)
+    return e["traffic"] if e else None
 
 
 _bwp = None
@@ -248,20 +254,111 @@ def oracle_sample(cfg, rows=256):
     app, W = cfg["app"], cfg["W"]
     if app == "hotspot":
         n = min(cfg["W"], 1024)
-        T, P = synth.hotspot(cfg["seed"], n, rows)
+        T, P = _sample_input(cfg, n, rows)
         prm = oracle.params("hotspot", n, rows, 1, cfg["scheme"], cfg["rate"], cfg["recon"])
         t0 = time.perf_counter()
         oracle.hotspot(prm, T, P, 1)
         return (n * rows) / (time.perf_counter() - t0), f"1 Hotspot step on a {n}x{rows} grid"
     u8 = app == "median"
-    img = synth.image(cfg["cls"], cfg["seed"], W, rows, np.uint8 if u8 else np.float32)
+    img = _sample_input(cfg, W, rows)
     prm = oracle.params(app, W, rows, cfg["r"], cfg["scheme"], cfg["rate"], cfg["recon"], 128 if u8 else 32)
     t0 = time.perf_counter()
     oracle.run(prm, img)
     return (W * rows) / (time.perf_counter() - t0), f"{W}x{rows} rows of one frame"
 
 
+def host_cores():
+    try:
+        return len(os.sched_getaffinity(0))
+    except Exception:
+        return os.cpu_count() or 1
+
+
+def cpu_model():
+    try:
+        for line in open("/proc/cpuinfo"):
+            if line.startswith("model name"):
+                return line.split(":", 1)[1].strip()
+    except Exception:
+        pass
+    return "unknown"
+
+
+_samples = {}
+
+
+def _sample_input(cfg, W, rows):
+    """the synthetic sample the CPU legs run on (generated once per shape)"""
+    import synth
+    key = (cfg["workload"], W, rows)
+    if key not in _samples:
+        if cfg["app"] == "hotspot":
+            _samples[key] = synth.hotspot(cfg["seed"], W, rows)
+        else:
+            _samples[key] = synth.image(cfg["cls"], cfg["seed"], W, rows,
+                                        np.uint8 if cfg["app"] == "median" else np.float32)
+    return _samples[key]
+
+
+def oracle_sample_bands(cfg, rows=256, threads=None, check=False):
+    """the same oracle, band-parallel over the host cores: the
+    sample's rows are cut into `threads` bands; each band runs oracle.run /
+    oracle.hotspot on its rows plus a halo in its own thread (the C oracle runs
+    without the GIL), and the band's own rows are kept.  Band starts are
+    aligned to the perforation period and the halo covers radius + rebuild
+    distance, so the stitched result equals the single-threaded run (check)."""
+    import concurrent.futures as cf
+
+    import oracle
+    import synth
+    threads = threads or host_cores()
+    app, W = cfg["app"], cfg["W"]
+    den = cfg["rate"][1]
+    align = int(np.lcm(den, 16))
+    r = 1 if app == "hotspot" else (3 if app == "gauss_sobel" else cfg["r"])
+    halo = -(-(r + den) // align) * align
+    per = -(-(-(-rows // threads)) // align) * align
+    cuts = list(range(0, rows, per)) + [rows]
+    if app == "hotspot":
+        n = min(W, 1024)
+        T, P = _sample_input(cfg, n, rows)
+        whole = lambda: oracle.hotspot(oracle.params("hotspot", n, rows, 1, cfg["scheme"], cfg["rate"],  # noqa: E731
+                                                     cfg["recon"]), T, P, 1)
+
+        def band(k):
+            a, b = max(0, cuts[k] - halo), min(rows, cuts[k + 1] + halo)
+            o = oracle.hotspot(oracle.params("hotspot", n, b - a, 1, cfg["scheme"], cfg["rate"], cfg["recon"]),
+                               np.ascontiguousarray(T[a:b]), np.ascontiguousarray(P[a:b]), 1)
+            return o[cuts[k] - a:cuts[k + 1] - a]
+        px, desc = n * rows, f"1 Hotspot step on a {n}x{rows} grid"
+    else:
+        u8 = app == "median"
+        img = _sample_input(cfg, W, rows)
+        G = 128 if u8 else 32
+        whole = lambda: oracle.run(oracle.params(app, W, rows, cfg["r"], cfg["scheme"], cfg["rate"],  # noqa: E731
+                                                 cfg["recon"], G), img)
+
+        def band(k):
+            a, b = max(0, cuts[k] - halo), min(rows, cuts[k + 1] + halo)
+            o = oracle.run(oracle.params(app, W, b - a, cfg["r"], cfg["scheme"], cfg["rate"], cfg["recon"], G),
+                           np.ascontiguousarray(img[a:b]))
+            return o[cuts[k] - a:cuts[k + 1] - a]
+        px, desc = W * rows, f"{W}x{rows} rows of one frame"
+    with cf.ThreadPoolExecutor(max_workers=threads) as ex:
+        t0 = time.perf_counter()
+        parts = list(ex.map(band, range(len(cuts) - 1)))
+        dt = time.perf_counter() - t0
+    same = None
+    if check:
+        # rows within halo of the sample's own top / bottom see the sample's border (both runs alike)
+        same = bool(np.array_equal(np.concatenate(parts), whole()))
+    return px / dt, desc, len(cuts) - 1, same
+
+
 def cpu_baseline(cfg, budget_s=10.0):
+    """the oracle as it stands on the box's host cores: single-threaded (the
+    headline CPU figure) and band-parallel over every core (same code, same
+    results), each on a bounded sample of about budget_s seconds"""
     px = 0.0
     t = 0.0
     n = 0
@@ -269,14 +366,29 @@ def cpu_baseline(cfg, budget_s=10.0):
     while t < budget_s and n < 200:
         rate, desc = oracle_sample(cfg)
         # rate = px/s for this call; accumulate time-weighted
-        dt = None
         px_call = cfg["W"] * 256 if cfg["app"] != "hotspot" else min(cfg["W"], 1024) * 256
-        dt = px_call / rate
         px += px_call
-        t += dt
+        t += px_call / rate
         n += 1
-    return {"value": px / t / 1e6, "unit": "Mpixel/s" if cfg["app"] != "hotspot" else "Mcell-updates/s",
-            "cores": 1, "kind": "oracle", "sample": f"{n} x oracle.run on {desc} ({t:.1f} s of CPU work)"}
+    unit = "Mpixel/s" if cfg["app"] != "hotspot" else "Mcell-updates/s"
+    cores = host_cores()
+    rows_mt = min(4096, max(1024, 128 * cores))  # >= 32-row bands, one per core
+    threads = max(1, min(cores, rows_mt // 32))
+    pxm, tm, nm, same = 0.0, 0.0, 0, None
+    while tm < budget_s / 2 and nm < 50:
+        rate, desc_mt, bands, ok = oracle_sample_bands(cfg, rows_mt, threads, check=(nm == 0))
+        if nm == 0:
+            same = ok
+        px_call = (cfg["W"] if cfg["app"] != "hotspot" else min(cfg["W"], 1024)) * rows_mt
+        pxm += px_call
+        tm += px_call / rate
+        nm += 1
+    return {"value": px / t / 1e6, "unit": unit, "cores": 1, "kind": "oracle",
+            "sample": f"{n} x oracle.run on {desc} ({t:.1f} s of CPU work)",
+            "cpu_model": cpu_model(), "nproc": cores,
+            "all_cores": {"value": pxm / tm / 1e6, "unit": unit, "cores": cores, "kind": "oracle, band-parallel",
+                          "sample": f"{nm} x {bands} bands of {desc_mt} on {threads} threads ({tm:.1f} s wall)",
+                          "identical_to_single_thread": same}}
 
 
 def run_reference(args, ws, rank):
@@ -298,7 +410,8 @@ def run_reference(args, ws, rank):
             "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "f64", "data": "synthetic",
             "config": {"workload": cfg["workload"], "sample": f"each step: oracle.run on {desc}"},
             "cpu_baseline": {"value": v, "unit": unit, "cores": 1, "kind": "oracle",
-                             "sample": f"{args.steps} steps of oracle.run on {desc}"},
+                             "sample": f"{args.steps} steps of oracle.run on {desc}", "cpu_model": cpu_model(),
+                             "nproc": host_cores()},
             "e2e": {"value": v, "unit": unit, "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
     print(json.dumps(line), flush=True)
 
@@ -312,6 +425,8 @@ def main():
     ap.add_argument("--config", default="C2", choices=sorted(CONFIGS))
     ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
     ap.add_argument("--no-variants", action="store_true")
+    ap.add_argument("--sweep", action="store_true",
+                    help="print only the C2 sweep (3 input classes x variants, incl. G = 1 px cells) as one JSON line")
     ap.add_argument("--no-cpu", action="store_true")
     ap.add_argument("--batch", type=int, default=0)
     ap.add_argument("--halo", default="nccl", choices=["nccl", "p2p"],
@@ -344,6 +459,10 @@ def main():
     es = 1 if u8 else 4
     unit = "Mpixel/s" if app != "hotspot" else "Mcell-updates/s"
 
+    if args.sweep:
+        if rank == 0:
+            print(json.dumps(bench_sweep(kp, stream, peak)), flush=True)
+        return
     if app == "hotspot":
         result = bench_hotspot(args, cfg, ws, rank, local, stream, peak, peak_src)
     else:
@@ -394,18 +513,24 @@ def main():
         algo_b = bytes_per_px(app, cfg["scheme"], cfg["rate"]) * px_step
         achieved = algo_b / (ms * 1e-3) / 1e9
         kkey = f"{app}{cfg['r']}_{cfg['scheme']}_{cfg['rate'][0]}-{cfg['rate'][1]}_{cfg['recon']}"
-        tr = ncu_traffic(kkey)
+        tr = ncu_traffic(args.config, kkey)
+        clk_sum = clk.summary()
         alu = None
-        if u8:  # the median is ALU-pipe bound: roofline on ALU lane-ops
-            # sorted-column network on 16-bit pairs, per 2 output pixels: column sort 6,
-            # combine 12 min/max, 3 one-column shifts + 1 unpack + 0.5 pack PRMT = 22.5 lane-ops
-            ops_px = 22.5 / 2
-            sm_mhz = 1965.0
-            alu_peak = 148 * 4 * 16 * sm_mhz * 1e6 / 1e12  # T lane-ops/s: 0.5 warp-inst/clk/SMSP
-            alu_ach = ops_px * px_step / (ms * 1e-3) / 1e12
-            alu = {"bound": "alu", "achieved": alu_ach, "peak": alu_peak, "unit": "Tlane-op/s",
-                   "frac": alu_ach / alu_peak, "ops_per_px": ops_px,
-                   "peak_derivation": "148 SM x 4 SMSP x 16 lanes/clk (ALU pipe, 1 warp-inst / 2 clk) x 1965 MHz"}
+        ent = ncu_entry(args.config, kkey)
+        if u8 and ent:  # the median is ALU-pipe bound: a pipe-resolved roofline
+            # achieved = ALU-pipe warp instructions of this launch (ncu, same launch configuration)
+            # / the launch's CUDA-event time; peak = the ALU pipe's issue rate, 0.5 warp-instruction
+            # per cycle per SM sub-partition (16 lanes/clk), x 4 x 148 at the SM clock sampled here
+            sm_mhz = clk_sum.get("sm_mhz") or 1965.0
+            alu_peak = 0.5 * 4 * 148 * sm_mhz * 1e6 / 1e9  # G warp-inst/s
+            alu_ach = ent["warp_inst_pipe_alu"] / (ms * 1e-3) / 1e9
+            alu = {"bound": "alu", "achieved": alu_ach, "peak": alu_peak, "unit": "Gwarp-inst/s (ALU pipe)",
+                   "frac": alu_ach / alu_peak, "traffic": tr, "kernel": kkey,
+                   "warp_inst_pipe_alu_per_launch": ent["warp_inst_pipe_alu"],
+                   "warp_inst_pipe_fma_per_launch": ent["warp_inst_pipe_fma"],
+                   "ncu_pipe_alu_pct_of_peak": ent["pipe_alu_pct_of_peak"],
+                   "peak_derivation": f"148 SM x 4 SMSP x 0.5 ALU warp-inst/clk x {sm_mhz:.0f} MHz (sampled)",
+                   "source": "profiles/ncu_traffic.json (tools/ncu_traffic.py)"}
         pmix = mixed_peak_gbs(x.data_ptr(), yex.data_ptr(), px_step * es, cfg["scheme"], cfg["rate"], G,
                               stream=stream.cuda_stream, pitch_bytes=W * es) if not u8 else None
         result = {
@@ -426,7 +551,7 @@ def main():
                          "algorithmic_bytes_per_launch": algo_b, "peak_source": peak_src,
                          "peak_mix": pmix, "frac_mix": achieved / pmix if pmix else None,
                          "peak_mix_source": "tools/bwprobe.cu on this box: plain stream, same read/write mix and CTA footprint"},
-            "clocks": clk.summary(),
+            "clocks": clk_sum,
             "gpu_launches": args.steps,
         }
         if alu:
@@ -643,6 +768,47 @@ def bench_c2_row_bands(kp, ws, rank, stream, steps):
             "parity": "ok" if min_over_ranks(ws, 1.0 if ok else 0.0) > 0 else "MISMATCH"}
 
 
+def bench_sweep(kp, stream, peak, steps=10):
+    """SURVEY 8(d) C2 sweep: the three synthetic input classes of Fig. 7
+    (flat / natural / pattern) x {Gaussian5, Sobel3} x every
+    row / column / checkerboard variant at 128-B cells, plus the pixel-granular
+    (G = 1) column and checkerboard variants the paper's ">= 32 B" rule
+     advises against.  Speedup vs the exact kernel on the same
+    frames, error vs the exact output (MRE; Sobel: ME)."""
+    import torch
+
+    import synth
+    cfg = CONFIGS["C2"]
+    W, H, B = cfg["W"], cfg["H"], cfg["batch"]
+    px = B * W * H
+    x = torch.empty((B, H, W), device="cuda")
+    y, yex = torch.empty_like(x), torch.empty_like(x)
+    out = []
+    for cls in ("flat", "natural", "pattern"):
+        synth.image_device(cls, synth.SEED_C2 + synth.CLASSES[cls], W, H, B, x.data_ptr(), False, stream.cuda_stream)
+        for app, r in (("gaussian", 2), ("sobel", 1)):
+            with kp.Plan(app, W, H, r, "none", (0, 1), "nn", batch=B) as ex:
+                ms_ex = time_kernel(lambda: ex.run(x, yex, stream), stream, steps, 3)
+            out.append({"class": cls, "app": app, "r": r, "scheme": "none", "rate": [0, 1], "recon": "-",
+                        "granule_bytes": None, "ms": ms_ex, "speedup": 1.0, "error": 0.0,
+                        "hbm_gbs": 8 * px / ms_ex / 1e6})
+            for scheme in ("row", "col", "checker"):
+                for gb in ((128,) if scheme == "row" else (128, 4)):
+                    for rate in ((1, 2), (1, 4), (3, 4)):
+                        for recon in ("nn", "li"):
+                            with kp.Plan(app, W, H, r, scheme, rate, recon, batch=B, granule_bytes=gb) as p:
+                                ms = time_kernel(lambda: p.run(x, y, stream), stream, steps, 3)
+                                err, _ = p.error(yex, y, stream)
+                            k = 1.0 if gb == 4 else 1.0 - rate[0] / rate[1]  # G = 1 px: every 32-B sector is read
+                            out.append({"class": cls, "app": app, "r": r, "scheme": scheme, "rate": list(rate),
+                                        "recon": recon, "granule_bytes": gb, "ms": ms, "speedup": ms_ex / ms,
+                                        "error": err, "hbm_gbs": bytes_per_px(app, scheme, rate) * px / ms / 1e6,
+                                        "frac": bytes_per_px(app, scheme, rate) * px / ms / 1e6 / peak,
+                                        "dram_bytes_floor_per_px": 4 * k + 4})
+    return {"sweep": out, "workload": "C2 sweep: 8 x 4096^2 fp32 frames per class, seeds SEED_C2 + class",
+            "metric": "ms per launch (CUDA events, 10 launches after 3 warm-up), speedup vs exact, error vs exact"}
+
+
 def bench_hotspot(args, cfg, ws, rank, local, stream, peak, peak_src):
     import torch
 
@@ -732,9 +898,17 @@ def bench_hotspot(args, cfg, ws, rank, local, stream, peak, peak_src):
                                  if args.halo == "p2p" else "NCCL send/recv per launch") if ws > 1 else "none")},
             "speedup_vs_exact": ms_ex / ms, "error": {"metric": "mre", "value": mre, "count": cnt},
             "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
-                         "frac": achieved / peak, "traffic": None, "peak_source": peak_src,
+                         "frac": achieved / peak,
+                         # per-step launch on one GPU (tools/ncu_traffic.py); blocked / banded runs: none captured
+                         "traffic": ncu_traffic("C4", f"hotspot1_{cfg['scheme']}_{cfg['rate'][0]}-{cfg['rate'][1]}_"
+                                                      f"{cfg['recon']}") if ws == 1 and args.tblock == 1 else None,
+                         "kernel": "hotspot per-step launch" if args.tblock == 1 else "hotspot_tb_kernel",
+                         "algorithmic_bytes_per_launch": algo_b / max(1, -(-iters // max(args.tblock, 1))),
+                         "peak_source": peak_src,
                          "peak_mix": pmix, "frac_mix": achieved / pmix if pmix else None},
-            "clocks": clk.summary(), "gpu_launches": args.steps * (-(-iters // args.tblock)) * (3 if ws > 1 and args.halo == "p2p" else 1),
+            # our kernels per timed call: one per launch of TBLOCK steps; banded runs split each launch into
+            # boundary rows (2 launches) + interior (PERF_KEY_OVERLAP), peer-store runs add signal + wait kernels
+            "clocks": clk.summary(), "gpu_launches": args.steps * (-(-iters // args.tblock)) * (3 if ws > 1 else 1),
             "temporal_blocking": tblock}
 
 

@@ -63,7 +63,7 @@ def _boundary_cols(W, tw):
     return sorted(x for x in xs if 0 <= x < W)
 
 
-def _check_frame(app, r, prm, img, got, W, H, tw, rows=True, cols=True, xstep=1):
+def _check_frame(app, r, prm, img, got, W, H, tw, rows=True, cols=True, xstep=1, max_strip_cols=None):
     if rows:  # (xstep coprime to the 16-column lane chunk still visits every lane position)
         ys = _boundary_rows(H)
         yy, xx = np.meshgrid(ys, np.arange(0, W, xstep), indexing="ij")
@@ -71,6 +71,8 @@ def _check_frame(app, r, prm, img, got, W, H, tw, rows=True, cols=True, xstep=1)
         assert_close(app, r, got[yy.ravel(), xx.ravel()], want)
     if cols:
         xs = _boundary_cols(W, tw)
+        if max_strip_cols:  # (the u8 frames are 8192 rows tall: the first strip boundary + the image edges)
+            xs = [x for x in xs if x < 2 or x >= W - 2 or abs(x - tw) <= 2][:max_strip_cols]
         xx, yy = np.meshgrid(xs, np.arange(H), indexing="ij")
         want = oracle.run_pixels(prm, img, xx.ravel(), yy.ravel())
         assert_close(app, r, got[yy.ravel(), xx.ravel()], want)
@@ -135,7 +137,8 @@ def test_c3_bench_launch(rate):
     prm = oracle.params("median", W, H, 1, "col", rate, "nn", G_BYTES)
     for f, rows, cols in ((0, True, False), (B - 1, False, True)):
         img = synth.image(cfg["cls"], cfg["seed"] + f, W, H, np.uint8)
-        _check_frame("median", 1, prm, img, y[f].cpu().numpy(), W, H, 2048, rows=rows, cols=cols, xstep=3)
+        _check_frame("median", 1, prm, img, y[f].cpu().numpy(), W, H, 2048, rows=rows, cols=cols, xstep=3,
+                     max_strip_cols=9)
 
 
 @pytest.mark.parametrize("scheme,rate,recon", [("row", (1, 2), "li"), ("row", (3, 4), "nn"), ("none", (0, 1), "nn")])
