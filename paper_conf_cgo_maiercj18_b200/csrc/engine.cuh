@@ -21,6 +21,8 @@
 //     results per row); outputs leave with 128-bit stores;
 //   * full/empty mbarriers per slot; consumer warps run independently.
 #pragma once
+#include <cuda.h>  // CUtensorMap
+
 #include <cstdint>
 
 #include "ptx.cuh"
@@ -29,9 +31,19 @@ namespace kp {
 
 enum { S_NONE = 0, S_ROW = 1, S_COL = 2, S_CHECKER = 3, S_STENCIL1 = 4 };
 enum { R_NN = 0, R_LI = 1 };
-enum { L_AUTO = 0, L_BULK = 1, L_ASYNC16 = 2, L_SCALAR = 3, L_RUNS = 4 };
+enum { L_AUTO = 0, L_BULK = 1, L_ASYNC16 = 2, L_SCALAR = 3, L_RUNS = 4, L_TMA = 5 };
+enum { TMA_NONE = 0, TMA_COL = 1, TMA_CHK = 2 };
 
 struct KParams {
+  // L_TMA (column scheme / keep-one checkerboard, fp32): the kept cells of a
+  // row arrive as ONE tensor-tile load into a packed ring slot (DESIGN.md
+  // "TMA cell loads").  TMA_COL: 3-D map {L = kept run of a den-cell group,
+  // group, row}, box {L, tma_ng, 1}; group g's run lands at (g - g0) * L.
+  // TMA_CHK: 3-D map {G, cell, row}, box {G, tma_ng * den, 1} traversed with
+  // stride den along the cells from the row's first kept cell (-y mod den):
+  // the kept cells land packed as the compact slots expect.
+  CUtensorMap tmap;  // host copy; the kernel reads its own __grid_constant__ parameter (kernel.cuh)
+  int tma_mode, tma_ng, tma_L, tma_rows_per_frame;
   const void* in;   // frame 0; element (x, y_global) at (y_global - in_row0) * W + x
   const void* in2;  // Hotspot power (same geometry as in), else nullptr
   void* out;        // frame 0; output row y_global at (y_global - out_row0) * W
@@ -244,7 +256,7 @@ __device__ __forceinline__ void issue_bulk_row(const KParams& p, const Mask& m, 
 // ring slot = g & (nr-1), fill phase = g >> log2(nr).
 template <typename T, int SCHEME, int NIN, int TW>
 __device__ __forceinline__ void producer(const KParams& p, const Mask& m, const RowPlan& rp, int x0, int frame,
-                                         int g0, uint64_t* full, uint64_t* empty, T* ring) {
+                                         int g0, uint64_t* full, uint64_t* empty, T* ring, const void* tmap) {
   constexpr int V = VT<T>::V;  // 16-B load chunk
   const int lane = threadIdx.x & 31;
   const int cx0 = max(x0 - p.hx, 0);
@@ -275,6 +287,30 @@ __device__ __forceinline__ void producer(const KParams& p, const Mask& m, const 
   const T* lane_src0 = in + cx0 + lane * V;
   const T* lane_src1 = in2 + cx0 + lane * V;
 
+  // L_TMA: the row's kept cells as one tensor-tile load per row (KParams tmap)
+  if constexpr ((SCHEME == S_COL || SCHEME == S_CHECKER) && NIN == 1 && sizeof(T) == 4) {
+    if (p.loader == L_TMA) {
+      // first loaded group: the one left of the strip (its last kept columns are
+      // the strip's apron); checkerboard: the compact slots' first cell (kperf.cu)
+      const int gg0 = x0 / (p.G * m.den) - 1;
+      const uint32_t bytes = (uint32_t)(p.tma_ng * p.tma_L * (int)sizeof(T));
+      if (lane == 0) tma_prefetch_desc(tmap);
+      for (int i = 0; i < rp.nload; ++i) {
+        const int g = g0 + i;
+        const int slot = g & (p.nr - 1);
+        if (g >= p.nr) mbar_wait(&empty[slot], ((g >> p.nr_log2) - 1) & 1);
+        const int y = row_of_idx<SCHEME>(m, rp, i);
+        const int row = frame * p.tma_rows_per_frame + (y - p.in_row0);
+        if (lane == 0) {
+          T* dst = ring + slot * slot_elems;
+          mbar_arrive_expect_tx(&full[slot], bytes);
+          if (SCHEME == S_COL) tma_load_3d(dst, tmap, 0, gg0, row, &full[slot]);
+          else tma_load_3d(dst, tmap, 0, gg0 * m.den + (m.den - y % m.den) % m.den, row, &full[slot]);
+        }
+      }
+      return;
+    }
+  }
   // compact keep-one checkerboard slots (kperf.cu chk_compact): a row keeps
   // cells c == -y mod den only, packed at ((c - (x0/G - den)) / den) * G, so
   // chunk k has one slot offset for every row that keeps it.  A loop of its

@@ -169,7 +169,18 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
   const ChunkInfo ce = make_chunk<SCHEME>(p, m, cex);
   // edge fragment: 0 inside the image, 1 left of column 0, 2 right of column W-1, 3 straddles W
   const int emode = (ex >= 0 && ex + EW <= p.W) ? 0 : (ex < 0 ? 1 : (ex == p.W ? 2 : 3));
-  const int ccol = xc - base, ecol = ex - base;
+  // ring column of global column x: x - base, or -- TMA column loads (kperf.cu
+  // L_TMA) -- the packed slot: the kept run of group g (den cells, L kept
+  // columns) at (g - gg0) * L; columns that are never loaded map to 0 (their
+  // values are never used: kept ? own : rebuilt selects)
+  auto ringcol = [&](int x) {
+    if (SCHEME != S_COL || p.tma_mode != TMA_COL) return x - base;
+    const int gw = p.G * m.den, rel = x - (x0 / gw - 1) * gw;
+    if (rel < 0) return 0;
+    const int k = rel / gw, q = rel - k * gw;
+    return (q < p.tma_L && k < p.tma_ng) ? k * p.tma_L + q : 0;
+  };
+  const int ccol = ringcol(xc), ecol = ringcol(ex);
   const T* ring2 = ring + p.row_elems;  // second input (Hotspot power)
   // Stencil1: lane edges that are tile borders take their halo from the tile itself
   const uint32_t hf = hedge | (SCHEME == S_STENCIL1
@@ -237,8 +248,8 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
     ColF z;
     z.kept = ci.col_kept;
     const bool hb = ci.xb >= 0;
-    z.ca = z.kept ? col : ci.xa - base;
-    z.cb = (z.kept || !hb) ? z.ca : ci.xb - base;
+    z.ca = z.kept ? col : ringcol(ci.xa);
+    z.cb = (z.kept || !hb) ? z.ca : ringcol(ci.xb);
     z.lim = hb ? ci.xa + ci.xb - 2 * fx : 2 * n;  // sample i takes a iff 2 i <= lim
     if (RECON == R_NN && !z.kept && z.lim >= 2 * (n - 1)) z.cb = z.ca;  // NN: all samples take a
     else if (RECON == R_NN && !z.kept && z.lim < 0) z.ca = z.cb;        // NN: all take b
@@ -638,7 +649,9 @@ __device__ __noinline__ void consumer_generic(const KParams& p, const Mask& m, c
 // output rows, strip of TW columns), strip fastest (the launcher sizes seg_h).
 template <class App, int SCHEME, int RECON, int NCW>
 __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : (NCW == 2 ? 6 : App::MINB))
-    perf_kernel(const __grid_constant__ KParams p) {
+    perf_kernel(const __grid_constant__ KParams p, const __grid_constant__ CUtensorMap tmap) {
+  // (the TMA descriptor is a kernel parameter of its own: its generic address,
+  // taken here, is what cp.async.bulk.tensor needs -- KParams::tmap is the host copy)
   using T = typename App::T;
   constexpr int V = App::V;
   constexpr int TW = NCW * 32 * V;
@@ -664,7 +677,7 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : (NCW
   const int nact = min(NCW, (p.W - x0 + 32 * V - 1) / (32 * V));
   if (threadIdx.x == 0) {
     for (int s = 0; s < p.nr; ++s) {
-      mbar_init(&full[s], (p.loader == L_BULK || p.loader == L_RUNS) ? 1u : 32u);
+      mbar_init(&full[s], (p.loader == L_BULK || p.loader == L_RUNS || p.loader == L_TMA) ? 1u : 32u);
       mbar_init(&empty[s], (uint32_t)(32 * nact));  // every consumer lane arrives
     }
     mbar_fence_init();
@@ -688,7 +701,7 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : (NCW
     const int ye = min(ys + p.seg_h, p.y_end);
     const RowPlan rp = make_row_plan<SCHEME>(p, m, ys, ye, App::VR);
     if (!p.inline_prod && warp == 0) {  // (Ia) data perforation: only kept samples leave HBM
-      producer<T, SCHEME, App::NIN, TW>(p, m, rp, x0, frame, g0, full, empty, ring);
+      producer<T, SCHEME, App::NIN, TW>(p, m, rp, x0, frame, g0, full, empty, ring, &tmap);
     } else {
       const int nv = n_recipes<SCHEME>(p, ys, ye, App::VR);
       __syncwarp();
@@ -782,7 +795,7 @@ cudaError_t launch_one(const KParams& p, unsigned grid, size_t smem, cudaStream_
     q.n_segs = (rows + q.seg_h - 1) / q.seg_h;
     grid = (unsigned)((long long)q.n_strips * q.n_segs * q.frames);
   }
-  k<<<grid, 32 * (NCW + (q.inline_prod ? 0 : 1)), smem, s>>>(q);
+  k<<<grid, 32 * (NCW + (q.inline_prod ? 0 : 1)), smem, s>>>(q, q.tmap);
   return cudaGetLastError();
 }
 

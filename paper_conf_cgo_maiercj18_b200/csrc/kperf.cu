@@ -1,6 +1,7 @@
 // kperf.cu -- the C ABI (include/kperf.h): plan validation, launch geometry,
 // Hotspot time loop (single device, banded with NCCL halo exchange, or banded
 // on one device for testing), error metric, host-buffer entry point.
+#include <cudaTypedefs.h>  // PFN_cuTensorMapEncodeTiled
 #include <cuda_runtime.h>
 #include <nccl.h>
 
@@ -138,10 +139,62 @@ static void hotspot_coeffs(float& sdc, float& rx1, float& ry1, float& rz1, float
   amb = 80.0f;
 }
 
-// Launch geometry for rows [y_begin, y_end) of `frames` frames.
+#ifndef KPERF_TMA
+#define KPERF_TMA 1  // auto loader: column / keep-one checkerboard cells by one TMA tensor-tile load per row
+#endif
+
+// cuTensorMapEncodeTiled through the runtime's driver entry point (no libcuda link)
+static PFN_cuTensorMapEncodeTiled_v12000 tma_encoder() {
+  static PFN_cuTensorMapEncodeTiled_v12000 fn = nullptr;
+  static bool tried = false;
+  if (!tried) {
+    tried = true;
+    void* f = nullptr;
+    cudaDriverEntryPointQueryResult q;
+    if (cudaGetDriverEntryPoint("cuTensorMapEncodeTiled", &f, cudaEnableDefault, &q) == cudaSuccess &&
+        q == cudaDriverEntryPointSuccess)
+      fn = reinterpret_cast<PFN_cuTensorMapEncodeTiled_v12000>(f);
+    else
+      cudaGetLastError();
+  }
+  return fn;
+}
+
+// the tensor map of a TMA cell load (KParams::tmap): fp32 rows of W, `rows`
+// rows (every frame's rows, pitch W), groups of den cells of G columns
+static bool encode_tma(KParams& k, const void* in, int W, long long rows) {
+  PFN_cuTensorMapEncodeTiled_v12000 enc = tma_encoder();
+  if (!enc) return false;
+  const cuuint64_t G = (cuuint64_t)k.G, den = (cuuint64_t)k.den, ng = (cuuint64_t)W / (G * den);
+  CUresult r;
+  if (k.tma_mode == kp::TMA_COL) {
+    const cuuint64_t dims[3] = {(cuuint64_t)k.tma_L, ng, (cuuint64_t)rows};
+    const cuuint64_t strides[2] = {G * den * 4, (cuuint64_t)W * 4};
+    const cuuint32_t box[3] = {(cuuint32_t)k.tma_L, (cuuint32_t)k.tma_ng, 1};
+    const cuuint32_t es[3] = {1, 1, 1};
+    r = enc(&k.tmap, CU_TENSOR_MAP_DATA_TYPE_FLOAT32, 3, const_cast<void*>(in), dims, strides, box, es,
+            CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_128B,
+            CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+  } else {  // {G, cell, row}, traversal stride den along the cells: every den-th cell from the start cell
+    const cuuint64_t dims[3] = {G, ng * den, (cuuint64_t)rows};
+    const cuuint64_t strides[2] = {G * 4, (cuuint64_t)W * 4};
+    const cuuint32_t box[3] = {(cuuint32_t)G, (cuuint32_t)(k.tma_ng * k.den), 1};
+    const cuuint32_t es[3] = {1, (cuuint32_t)k.den, 1};
+    r = enc(&k.tmap, CU_TENSOR_MAP_DATA_TYPE_FLOAT32, 3, const_cast<void*>(in), dims, strides, box, es,
+            CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_128B,
+            CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
+  }
+  if (getenv("KPERF_TMA_DEBUG"))
+    fprintf(stderr, "tma mode %d G %d den %d L %d ng %d W %d rows %lld in %p -> %d\n", k.tma_mode, k.G, k.den, k.tma_L,
+            k.tma_ng, W, rows, in, (int)r);
+  return r == CUDA_SUCCESS;
+}
+
+// Launch geometry for rows [y_begin, y_end) of `frames` frames (input frame
+// pitch: in_frame_rows rows of W, default H).
 static perf_status make_params(const perf_plan_s* P, const void* in, const void* in2, void* out, int frames,
                                int in_row0, int avail0, int avail1, int out_row0, int y_begin, int y_end,
-                               KParams& k, unsigned& grid, size_t& smem) {
+                               KParams& k, unsigned& grid, size_t& smem, int in_frame_rows = -1) {
   const int es = (int)elem_size(P->app);
   const int CV = 16 / es;  // elements per 16-B chunk (load / store / alignment unit)
   // elements per consumer lane per row (must match App::V in apps.cuh)
@@ -158,7 +211,7 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   k.in = in;
   k.in2 = in2;
   k.out = out;
-  k.in_fstride = (long long)P->W * P->H;
+  k.in_fstride = (long long)P->W * (in_frame_rows > 0 ? in_frame_rows : P->H);
   k.out_fstride = (long long)P->W * P->H;
   k.W = P->W;
   k.ncw = NCW;
@@ -191,7 +244,9 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   // TMA bulk runs of kept cells: cells of whole 16-B chunks, <= 64 cells per tile row (2 run slots per lane)
   const bool runs_ok = k.vec_io && chunk_uniform && (scheme == PERF_SCHEME_COL || scheme == PERF_SCHEME_CHECKER) &&
                        (TW + 2 * ((CV + k.den * k.G + CV - 1) / CV) * CV) / k.G + 2 <= 64;
-  int loader = (int)P->loader;
+  // (an explicit TMA request starts as the cp.async cell loader: the slot layout
+  // below is chosen for it, then the TMA block switches the loader or refuses)
+  int loader = P->loader == kp::L_TMA ? (int)kp::L_ASYNC16 : (int)P->loader;
   if (loader == kp::L_AUTO) {
     if (!k.vec_io) loader = kp::L_SCALAR;
     else if (rowwise) loader = kp::L_BULK;
@@ -231,6 +286,47 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
     k.chk_compact = 1;
     k.row_elems = compact_elems;
   }
+  // TMA cell loads (fp32, one input, every warp on the fast path): the row's kept
+  // cells as one tensor-tile load into a packed slot (engine.cuh producer,
+  // kernel.cuh ringcol).  Column scheme: every group of den cells keeps a run of
+  // L = (den - num) G columns (skip-one: phases 0..den-2, keep-one: phase 0); the
+  // slot holds the strip's groups + one group each side.  Keep-one checkerboard:
+  // the compact slots above, one cell per group.  Any shape that does not fit
+  // keeps the 16-B cp.async loader.
+  k.tma_mode = kp::TMA_NONE;
+  {
+    const bool want = P->loader == kp::L_TMA || (P->loader == kp::L_AUTO && KPERF_TMA && loader == kp::L_ASYNC16);
+    const int gw = k.G * k.den;
+    const bool common = es == 4 && nin_of(P->app) == 1 && k.fast_ok && k.vec_io && k.vec32 && P->W % (32 * V) == 0 &&
+                        k.den > 1 && gw > 0 && TW % gw == 0 && P->W % gw == 0 && (k.G * es) % 16 == 0 && in != nullptr;
+    int mode = kp::TMA_NONE, L = 0, ng = 0;
+    if (want && common && scheme == PERF_SCHEME_COL) {
+      L = (k.den - k.num) * k.G;
+      ng = TW / gw + 2;
+      if (L <= 256 && ng <= 256) mode = kp::TMA_COL;
+    } else if (want && common && scheme == PERF_SCHEME_CHECKER && k.chk_compact && (TW / k.G) % k.den == 0) {
+      L = k.G;
+      ng = k.row_elems / k.G;
+      if (L <= 256 && ng * k.den <= 256) mode = kp::TMA_CHK;
+    }
+    if (mode != kp::TMA_NONE) {
+      k.tma_mode = mode;
+      k.tma_L = L;
+      k.tma_ng = ng;
+      k.tma_rows_per_frame = (int)(k.in_fstride / P->W);
+      if (encode_tma(k, in, P->W, (long long)frames * k.tma_rows_per_frame)) {
+        k.loader = loader = kp::L_TMA;
+        if (mode == kp::TMA_COL) k.row_elems = ng * L;
+        k.row_elems = (k.row_elems + 31) / 32 * 32;  // tensor-tile destinations: 128-B aligned slots
+      } else {
+        k.tma_mode = kp::TMA_NONE;
+      }
+    }
+    if (P->loader == kp::L_TMA && k.loader != kp::L_TMA)
+      return fail(PERF_ERR_UNSUPPORTED,
+                  "loader TMA needs fp32 column / keep-one checkerboard cells, W a multiple of 256 and of den * G, "
+                  "aligned buffers and a driver with cuTensorMapEncodeTiled");
+  }
   // ring: rows a consumer holds for reconstruction + prefetch depth
   int hold = 1;
   if (scheme == PERF_SCHEME_ROW) hold = 2;
@@ -240,7 +336,9 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   const int nin = P->app == PERF_APP_HOTSPOT ? 2 : 1;
   const size_t slot_bytes = (size_t)k.row_elems * nin * es;
   auto bar_bytes = [](int n) { return (size_t)((2 * n * 8 + 127) & ~127); };
-  int seg = (int)(P->tile_h > 0 ? P->tile_h : 128);
+  // segment cap (the launcher then picks the wave-filling height below it): Hotspot
+  // 64 rows -- its two-input slots + 32-B recipes for 134 rows would leave 2 CTAs/SM
+  int seg = (int)(P->tile_h > 0 ? P->tile_h : (nin == 2 ? 64 : 128));
   if (s1) seg = (seg + k.tile1_h - 1) / k.tile1_h * k.tile1_h;  // whole Stencil1 tiles per segment
   // recipes per segment: seg + 2 VR rows, Stencil1: every tile restarts its window
   k.nrec = s1 ? seg + (seg / k.tile1_h + 1) * 2 * kp::kMaxVR : seg + 2 * kp::kMaxVR;
@@ -419,7 +517,7 @@ perf_status perf_plan_set(perf_plan_t p, int key, long long v) {
       p->metric = v;
       return PERF_OK;
     case PERF_KEY_LOADER:
-      if (v < 0 || v > 4) return fail(PERF_ERR_INVALID_ARG, "bad LOADER");
+      if (v < 0 || v > 5) return fail(PERF_ERR_INVALID_ARG, "bad LOADER");
       p->loader = v;
       return PERF_OK;
     case PERF_KEY_RING:
@@ -1279,9 +1377,8 @@ perf_status perf_run_band(perf_plan_t p, void* in_band, void* out, void* stream)
   unsigned grid;
   size_t smem;
   st = make_params(p, in_band, nullptr, out, (int)p->batch, y0 - hb, std::max(0, y0 - hb), std::min(Hg, y0 + h + hb), y0,
-                   y0, y0 + h, k, grid, smem);
+                   y0, y0 + h, k, grid, smem, hp.buf_rows);
   if (st != PERF_OK) return st;
-  k.in_fstride = (long long)fin;
   k.out_fstride = (long long)h * p->W;
   cudaError_t e = dispatch(p, k, grid, smem, s);
   if (e != cudaSuccess) return cuda_fail(e, "perf_run_band launch");

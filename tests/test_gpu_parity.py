@@ -660,3 +660,60 @@ def test_median_col_nn_cell_lanes(gbytes, rate):
     pat = synth.image("pattern", 0x5EED2500, W, H, np.uint8)  # high-frequency: every window differs
     got = gpu_run("median", 1, pat, "col", rate, "nn", G_bytes=gbytes, batch=1)
     assert_close("median", 1, got, oracle.run(oracle.params("median", W, H, 1, "col", rate, "nn", gbytes), pat))
+
+
+@pytest.mark.parametrize("app,r", [("gaussian", 2), ("sobel", 1), ("gauss_sobel", 2), ("inversion", 0)])
+@pytest.mark.parametrize("scheme,rate", [("col", (1, 2)), ("col", (1, 4)), ("col", (3, 4)), ("col", (1, 8)),
+                                         ("col", (7, 8)), ("checker", (1, 2)), ("checker", (3, 4)),
+                                         ("checker", (7, 8))])
+@pytest.mark.parametrize("gbytes", [32, 128])
+def test_tma_cell_loads(app, r, scheme, rate, gbytes):
+    """TMA tensor-tile cell loads (loader 5, the auto choice for fp32 column and
+    keep-one checkerboard cells): bit-identical to the 16-B cp.async loader
+    (loader 2, full-width / compact slots) and == the oracle; two 1024-column
+    strips and a third, 3 row segments, batch 2"""
+    W, H, B = 3072, 300, 2
+    imgs = np.stack([synth.image("natural", 0x5EED2600 + b, W, H) for b in range(B)])
+    for recon in ("nn", "li"):
+        tma = gpu_run(app, r, imgs, scheme, rate, recon, G_bytes=gbytes, batch=B, loader=5)
+        ref = gpu_run(app, r, imgs, scheme, rate, recon, G_bytes=gbytes, batch=B, loader=2)
+        assert np.array_equal(tma, ref), (recon,)
+        auto = gpu_run(app, r, imgs, scheme, rate, recon, G_bytes=gbytes, batch=B)
+        assert np.array_equal(auto, ref)
+    want = oracle.run(oracle.params(app, W, H, r, scheme, rate, "li", gbytes // 4), imgs[1])
+    assert_close(app, r, tma[1], want)
+
+
+def test_tma_loader_refuses_unsupported_shapes():
+    """loader 5 on shapes the tensor-tile path does not cover: a clear error,
+    and the auto loader silently keeps cp.async (results unchanged)"""
+    img = synth.image("natural", 7, 1100, 64)
+    for scheme, rate in (("col", (1, 2)), ("checker", (1, 4)), ("row", (1, 2))):
+        with pytest.raises(kp.PerfError):
+            gpu_run("gaussian", 2, img, scheme, rate, "li", loader=5)
+    got = gpu_run("gaussian", 2, img, "col", (1, 2), "li", G_bytes=128)
+    want = oracle.run(oracle.params("gaussian", 1100, 64, 2, "col", (1, 2), "li", 32), img)
+    assert_close("gaussian", 2, got, want)
+
+
+def test_tma_cell_loads_in_row_bands():
+    """perf_run_band with TMA cell loads (the frame pitch of the band buffer is
+    buf_rows): bands == the whole image"""
+    W, H, B = 2048, 200, 2
+    imgs = np.stack([synth.image("natural", 0x5EED2700 + b, W, H) for b in range(B)])
+    x = torch.from_numpy(imgs).cuda()
+    whole = torch.empty_like(x)
+    for scheme, rate in (("col", (1, 2)), ("checker", (3, 4))):
+        with kp.Plan("gaussian", W, H, 2, scheme, rate, "li", batch=B, loader=5) as p:
+            p.run(x, whole)
+        for k, (y0, h) in enumerate(((0, 90), (90, 110))):
+            with kp.Plan("gaussian", W, h, 2, scheme, rate, "li", batch=B, global_h=H, band_y0=y0, loader=5) as p:
+                hp = kp.perf_band_halo(p.handle, k, 2)
+                hb = hp["halo_rows"]
+                buf = torch.full((B, hp["buf_rows"], W), float("nan"), device="cuda")
+                lo, hi = max(0, y0 - hb), min(H, y0 + h + hb)
+                buf[:, lo - (y0 - hb):hi - (y0 - hb)] = x[:, lo:hi]
+                out = torch.empty((B, h, W), device="cuda")
+                kp.perf_run_band(p.handle, buf, out)
+                torch.cuda.synchronize()
+            assert torch.equal(out, whole[:, y0:y0 + h]), (scheme, k)

@@ -25,6 +25,13 @@ SETS = {
 }
 SETS["row34"] = [("gaussian", 2, "row", 3, 4, "nn"), ("gaussian", 2, "row", 3, 4, "li"), ("sobel", 1, "row", 3, 4, "nn"),
                  ("sobel", 1, "row", 3, 4, "li"), ("gaussian", 2, "none", 0, 1, "nn"), ("sobel", 1, "none", 0, 1, "nn")]
+SETS["hotspot"] = [("hotspot", 1, "none", 0, 1, "nn"), ("hotspot", 1, "row", 1, 2, "li"), ("hotspot", 1, "row", 1, 2, "nn")]
+SETS["colchk"] = [("gaussian", 2, "col", 1, 2, "li"), ("gaussian", 2, "col", 1, 2, "nn"), ("gaussian", 2, "col", 1, 4, "li"),
+                  ("gaussian", 2, "col", 1, 4, "nn"), ("gaussian", 2, "col", 3, 4, "li"), ("gaussian", 2, "col", 3, 4, "nn"),
+                  ("gaussian", 2, "checker", 1, 2, "li"), ("gaussian", 2, "checker", 1, 2, "nn"),
+                  ("gaussian", 2, "checker", 3, 4, "li"), ("gaussian", 2, "checker", 3, 4, "nn"),
+                  ("sobel", 1, "col", 1, 2, "nn"), ("sobel", 1, "col", 1, 4, "li"), ("sobel", 1, "checker", 3, 4, "li"),
+                  ("gaussian", 2, "none", 0, 1, "nn")]
 SETS["all"] = SETS["row"] + SETS["col"] + SETS["checker"]
 
 CHILD = r'''
@@ -52,6 +59,21 @@ def buf(app, shape=None):
     return (W, H, B) + bufs[k]
 for v in vs:
     app, r, sch, num, den, rc = v[:6]
+    if app == "hotspot":  # 16384^2, 20 steps per call
+        W = H = 16384
+        if "hs" not in bufs:
+            T = torch.empty((H, W), device="cuda"); P = torch.empty_like(T)
+            synth.hotspot_device(0x5EED0030, W, H, T.data_ptr(), P.data_ptr())
+            bufs["hs"] = (T, P, torch.empty_like(T))
+        T, P, O = bufs["hs"]
+        with kp.Plan(app, W, H, 1, sch, (num, den), rc, iters=20, **KEYS) as p:
+            p.hotspot(T, P, O)
+            e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+            e0.record()
+            for _ in range(3): p.hotspot(T, P, O)
+            e1.record(); e1.synchronize()
+            out["/".join(map(str, v))] = e0.elapsed_time(e1) / 3 / 20
+        continue
     W, H, B, x, y = buf(app, v[6:] or None)
     with kp.Plan(app, W, H, r, sch, (num, den), rc, batch=B, **KEYS) as p:
         for _ in range(3): p.run(x, y)
