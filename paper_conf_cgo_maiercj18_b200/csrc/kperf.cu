@@ -184,9 +184,6 @@ static bool encode_tma(KParams& k, const void* in, int W, long long rows) {
             CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_128B,
             CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
   }
-  if (getenv("KPERF_TMA_DEBUG"))
-    fprintf(stderr, "tma mode %d G %d den %d L %d ng %d W %d rows %lld in %p -> %d\n", k.tma_mode, k.G, k.den, k.tma_L,
-            k.tma_ng, W, rows, in, (int)r);
   return r == CUDA_SUCCESS;
 }
 
