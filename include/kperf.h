@@ -123,8 +123,13 @@ enum {
                                   per (buffers, plan state) into a CUDA graph and replayed (one launch per
                                   call); 0 = eager launches.  Peer-store (P2P) plans always run eagerly.
                                   Reads 2 after a capture failed and the plan fell back to eager launches */
-  PERF_KEY_EXCHANGE = 20       /* MEASUREMENT ONLY: 0 skips every halo exchange of banded runs (results are
+  PERF_KEY_EXCHANGE = 20,      /* MEASUREMENT ONLY: 0 skips every halo exchange of banded runs (results are
                                   then wrong at band edges) so the exchange's share of a step can be timed */
+  PERF_KEY_FOLD = 21           /* row scheme, fp32 Gaussian / Sobel / Gauss-Sobel, one kept row per period (den 2
+                                  or keep-one den 4): 1 (default) = the rebuild is folded into the vertical pass
+                                  -- per kept row one horizontal pass, each output row a compile-time weighted
+                                  sum of kept rows; 0 = rebuild every row,
+                                  then filter.  Same values (bit-identical on integer-valued inputs) */
 };
 
 /* size of a perf_p2p_export handle */

@@ -12,6 +12,7 @@
 // Border handling is clamp-to-edge on the rebuilt image (R8).
 #pragma once
 #include "engine.cuh"
+#include "fold.cuh"
 
 #ifndef KPERF_ULI
 #define KPERF_ULI 0
@@ -80,6 +81,53 @@ __device__ __forceinline__ f2 deriv_pair(const float* x) {
   return fma2(splat2(2.f), pk2(x[3] - x[1], x[4] - x[2]), sub2(pk2(x[4], x[5]), pk2(x[0], x[1])));
 }
 
+// vertical taps of the folded apps (fold.cuh)
+template <int R>
+struct BinomTaps;  // binomial smoothing, optionally scaled
+template <>
+struct BinomTaps<1> {
+  static constexpr float v[3] = {1.f, 2.f, 1.f};
+  static constexpr float g[3] = {1.f / 16, 2.f / 16, 1.f / 16};  // Gaussian 3x3 incl. its 1/16
+};
+template <>
+struct BinomTaps<2> {
+  static constexpr float v[5] = {1.f, 4.f, 6.f, 4.f, 1.f};
+  static constexpr float g[5] = {1.f / 256, 4.f / 256, 6.f / 256, 4.f / 256, 1.f / 256};
+};
+template <int R>
+struct DerivTaps;
+template <>
+struct DerivTaps<1> {
+  static constexpr float v[3] = {-1.f, 0.f, 1.f};
+};
+template <>
+struct DerivTaps<2> {
+  static constexpr float v[5] = {-1.f, -2.f, 0.f, 2.f, 1.f};
+};
+
+// output pair j of a folded row: sum over kept rows t of w(PH, t) * ring[slot(t)][j]
+// (compile-time weights of table TAB, kept rows relative to the arrival U)
+template <const FoldTab& TAB, int TMAX, int RK, int U, int PH, int NJ>
+__device__ __forceinline__ f2 fold_dot(const f2 (&ring)[8][NJ], int j) {
+  f2 acc = splat2(0.f);
+  static_for<0, 2 * kFoldT + 1>([&](auto tc) {
+    constexpr int t = decltype(tc)::value - kFoldT;
+    constexpr float w = TAB.w[PH][t + kFoldT];
+    if constexpr (w != 0.f) acc = fma2(splat2(w), ring[fold_slot<RK>(U, t - TMAX)][j], acc);
+  });
+  return acc;
+}
+template <const FoldTab& TAB, int TMAX, int RK, int U, int PH>
+__device__ __forceinline__ float fold_dot1(const float (&ring)[8]) {
+  float acc = 0.f;
+  static_for<0, 2 * kFoldT + 1>([&](auto tc) {
+    constexpr int t = decltype(tc)::value - kFoldT;
+    constexpr float w = TAB.w[PH][t + kFoldT];
+    if constexpr (w != 0.f) acc = fmaf(w, ring[fold_slot<RK>(U, t - TMAX)], acc);
+  });
+  return acc;
+}
+
 // ---------------------------------------------------------------------------
 template <int R>
 struct AppGauss {  // K1 Gaussian, binomial (2R+1)^2, fp32
@@ -89,6 +137,32 @@ struct AppGauss {  // K1 Gaussian, binomial (2R+1)^2, fp32
   static constexpr int V = 8, EW = 2, VR = R, NIN = 1, NWIN = 2 * R + 1, MINB = 4;
   f2 h[NWIN][V / 2];  // horizontal results, column pairs (FADD2/FFMA2 vertical pass)
   __device__ void init(const KParams&) {}
+  // folded row scheme (fold.cuh): vertical binomial taps incl. the 1/16, 1/256 scale
+  static constexpr bool FOLD = true;
+  template <int DEN, int RECON>
+  struct Fold {
+    static constexpr FoldTab tab = fold_tab<DEN, RECON>(BinomTaps<R>::g);
+    static constexpr FoldTab tabs[1] = {tab};
+    static constexpr FoldSched<DEN> sch = fold_sched<DEN>(tabs, 1);
+    static_assert(fold_sched_ok(sch), "fold schedule");
+  };
+  f2 fk[8][V / 2];  // kept rows' horizontal results, ring
+  template <int S>
+  __device__ __forceinline__ void fold_h(const Frag<float, V>& c, const Frag<float, EW>& e, int lane, uint32_t hf) {
+    float x[V + 2 * R];
+    ext_row<R, EW, V>(c, e, lane, hf, x);
+#pragma unroll
+    for (int j = 0; j < V / 2; ++j) fk[S][j] = smooth_pair<R>(x + 2 * j);
+  }
+  template <class F, int RK, int U, int PH, class Store>
+  __device__ __forceinline__ void fold_emit(int q, int ys, int ye, int, int, const KParams&, Store&& st) {
+    if (q < ys || q >= ye) return;
+    Frag<float, V> o;
+#pragma unroll
+    for (int j = 0; j < V / 2; ++j)
+      up2(fold_dot<F::tab, F::sch.tmax[PH], RK, U, PH, V / 2>(fk, j), o.v[2 * j], o.v[2 * j + 1]);
+    st(o);
+  }
   template <int U>
   __device__ __forceinline__ Frag<float, V> row(const Frag<float, V>& c, const Frag<float, EW>& e,
                                                 const Frag<float, V>&, int lane, uint32_t hf, int, int, const KParams&) {
@@ -120,6 +194,42 @@ struct AppSobel {  // K5 Sobel, |(Gx, Gy)|, fp32
   static constexpr int V = 8, EW = 2, VR = R, NIN = 1, NWIN = 2 * R + 1, MINB = R == 1 ? 4 : 3;
   f2 sx[NWIN][V / 2], dx[NWIN][V / 2];  // horizontal smoothing / derivative, column pairs
   __device__ void init(const KParams&) {}
+  // folded row scheme (fold.cuh): gx = vertical smoothing of dx, gy = vertical derivative of sx
+  static constexpr bool FOLD = true;
+  template <int DEN, int RECON>
+  struct Fold {
+    static constexpr FoldTab tx = fold_tab<DEN, RECON>(BinomTaps<R>::v);
+    static constexpr FoldTab ty = fold_tab<DEN, RECON>(DerivTaps<R>::v);
+    static constexpr FoldTab tabs[2] = {tx, ty};
+    static constexpr FoldSched<DEN> sch = fold_sched<DEN>(tabs, 2);
+    static_assert(fold_sched_ok(sch), "fold schedule");
+  };
+  f2 fs[8][V / 2], fd[8][V / 2];  // kept rows' horizontal smoothing / derivative, ring
+  template <int S>
+  __device__ __forceinline__ void fold_h(const Frag<float, V>& c, const Frag<float, EW>& e, int lane, uint32_t hf) {
+    float x[V + 2 * R];
+    ext_row<R, EW, V>(c, e, lane, hf, x);
+#pragma unroll
+    for (int j = 0; j < V / 2; ++j) {
+      fs[S][j] = smooth_pair<R>(x + 2 * j);
+      fd[S][j] = deriv_pair<R>(x + 2 * j);
+    }
+  }
+  template <class F, int RK, int U, int PH, class Store>
+  __device__ __forceinline__ void fold_emit(int q, int ys, int ye, int, int, const KParams&, Store&& st) {
+    if (q < ys || q >= ye) return;
+    Frag<float, V> o;
+#pragma unroll
+    for (int j = 0; j < V / 2; ++j) {
+      const f2 gx = fold_dot<F::tx, F::sch.tmax[PH], RK, U, PH, V / 2>(fd, j);
+      const f2 gy = fold_dot<F::ty, F::sch.tmax[PH], RK, U, PH, V / 2>(fs, j);
+      float m0, m1;
+      up2(fma2(gx, gx, mul2(gy, gy)), m0, m1);
+      o.v[2 * j] = sqrt_approx(m0);
+      o.v[2 * j + 1] = sqrt_approx(m1);
+    }
+    st(o);
+  }
   template <int U>
   __device__ __forceinline__ Frag<float, V> row(const Frag<float, V>& c, const Frag<float, EW>& e,
                                                 const Frag<float, V>&, int lane, uint32_t hf, int, int, const KParams&) {
@@ -161,6 +271,7 @@ struct AppInversion {  // K2 Inversion, 255 - x
   static constexpr bool ULI = KPERF_ULI;
   static constexpr bool IPROD = KPERF_IPROD;
   static constexpr int V = 8, EW = 2, VR = 0, NIN = 1, NWIN = 1, MINB = 4;
+  static constexpr bool FOLD = false;
   __device__ void init(const KParams&) {}
   template <int U>
   __device__ __forceinline__ Frag<float, V> row(const Frag<float, V>& c, const Frag<float, EW>&,
@@ -179,6 +290,7 @@ struct AppHotspot {
   static constexpr bool ULI = KPERF_ULI;
   static constexpr bool IPROD = KPERF_IPROD;
   static constexpr int V = 8, EW = 2, VR = 1, NIN = 2, NWIN = 3, MINB = 4;
+  static constexpr bool FOLD = false;
   float tc[3][V], tl[3], tr[3], pc[3][V];
   float sdc, rx1, ry1, rz1, amb;
   __device__ void init(const KParams& p) {
@@ -240,6 +352,68 @@ struct AppGaussSobel {
   f2 acc[4][V / 2];  // Gaussian rows in flight (x 256), lane columns, pairs; slot q % 4
   float acce[4];     // the same for the lane's edge column (xc - 1 / xc + V)
   f2 sr[2][V / 2], dr[2][V / 2];  // Sobel horizontal smoothing / derivative of Gaussian rows, slot q % 2
+  // folded row scheme (fold.cuh): Gaussian rows from the kept rows' horizontal
+  // results (the Gaussian taps over rebuilt rows folded into kept-row weights);
+  // the Sobel stage then runs on every Gaussian row as above (interior rows:
+  // no top / bottom clamp)
+  static constexpr bool FOLD = true;
+  template <int DEN, int RECON>
+  struct Fold {
+    static constexpr FoldTab tab = fold_tab<DEN, RECON>(BinomTaps<2>::g);
+    static constexpr FoldTab tabs[1] = {tab};
+    static constexpr FoldSched<DEN> sch = fold_sched<DEN>(tabs, 1);
+    static_assert(fold_sched_ok(sch), "fold schedule");
+  };
+  f2 fk[8][V / 2];  // kept rows' horizontal Gaussian, ring
+  float fke[8];     // ... of the lane's edge column
+  template <int S>
+  __device__ __forceinline__ void fold_h(const Frag<float, V>& c, const Frag<float, EW>& e, int lane, uint32_t) {
+    float x[V + 4];
+    ext_row<2, EW, V>(c, e, lane, 0u, x);
+#pragma unroll
+    for (int j = 0; j < V / 2; ++j) fk[S][j] = smooth_pair<2>(x + 2 * j);
+    float t[5];
+    if (lane < 16) { t[0] = e.v[1]; t[1] = e.v[2]; t[2] = e.v[3]; t[3] = c.v[0]; t[4] = c.v[1]; }
+    else { t[0] = c.v[V - 2]; t[1] = c.v[V - 1]; t[2] = e.v[0]; t[3] = e.v[1]; t[4] = e.v[2]; }
+    fke[S] = smooth<2>(t);
+  }
+  // Gaussian row q (ys - 1 <= q <= ye); Sobel output row q - 1 once q - 1 >= ys
+  template <class F, int RK, int U, int PH, class Store>
+  __device__ __forceinline__ void fold_emit(int q, int ys, int ye, int lane, int xc, const KParams& p, Store&& st) {
+    if (q < ys - 1 || q > ye) return;
+    constexpr int SQ = PH % 2, SM = (PH + 1) % 2;  // Sobel ring slots of rows q (and q - 2), q - 1 (DEN even)
+    float g[V + 2];
+#pragma unroll
+    for (int j = 0; j < V / 2; ++j)
+      up2(fold_dot<F::tab, F::sch.tmax[PH], RK, U, PH, V / 2>(fk, j), g[2 * j + 1], g[2 * j + 2]);
+    const float gve = fold_dot1<F::tab, F::sch.tmax[PH], RK, U, PH>(fke);
+    float gl = __shfl_up_sync(FULLMASK, g[V], 1);
+    float gright = __shfl_down_sync(FULLMASK, g[1], 1);
+    if (lane == 0) gl = gve;
+    if (lane == 31) gright = gve;
+    g[0] = gl;
+    g[V + 1] = gright;
+    if (xc <= 0) g[0] = g[1];
+    const int cl = p.W - 1 - xc;
+    if (cl < V) {
+#pragma unroll
+      for (int k = 1; k < V + 2; ++k) g[k] = k > cl + 1 ? g[k - 1] : g[k];
+    }
+    Frag<float, V> o;
+#pragma unroll
+    for (int j = 0; j < V / 2; ++j) {
+      const f2 sq = smooth_pair<1>(g + 2 * j), dq = deriv_pair<1>(g + 2 * j);
+      const f2 gx = fma2(splat2(2.f), dr[SM][j], add2(dr[SQ][j], dq));
+      const f2 gy = sub2(sq, sr[SQ][j]);
+      sr[SQ][j] = sq;
+      dr[SQ][j] = dq;
+      float m0, m1;
+      up2(fma2(gx, gx, mul2(gy, gy)), m0, m1);
+      o.v[2 * j] = sqrt_approx(m0);
+      o.v[2 * j + 1] = sqrt_approx(m1);
+    }
+    if (q >= ys + 1) st(o);
+  }
   __device__ void init(const KParams&) {
 #pragma unroll
     for (int k = 0; k < 4; ++k) {
@@ -348,6 +522,7 @@ struct AppMedian {
   // (kernel.cuh MEDC) leave the kept warps as the critical path; more resident
   // CTAs hide their latency (C3 col 1/2 NN 235 -> 196 us, exact 230 -> 228 us)
   static constexpr int V = 16, EW = 4, VR = 1, NIN = 1, NWIN = 3, MINB = 4;
+  static constexpr bool FOLD = false;
   static constexpr int NW = V / 2 + 2;  // 16-bit-pair words per row incl. the two halo words
   uint32_t r[3][NW];  // word 0 = (_, col -1), words 1..V/2 = cols 0..V-1, last = (col V, _)
   __device__ void init(const KParams&) {}

@@ -63,6 +63,7 @@ struct KParams {
                              // ((c - (x0/G - den)) / den) * G (kperf.cu: fast path for every warp)
   int fast_ok;               // every V-chunk lies in one mask cell (G % V == 0 or row scheme)
   int cellmap;               // median column NN: cell-grouped lanes (kernel.cuh MEDC)
+  int fold;                  // row scheme: rebuild folded into the vertical pass (fold.cuh), interior segments
   int vec_io;                // W % V == 0 and 16-B aligned buffers
   int vec32;                 // 32-B aligned lane chunks of the output (256-bit stores)
   int tile1_w, tile1_h;      // Stencil1 work-group tile

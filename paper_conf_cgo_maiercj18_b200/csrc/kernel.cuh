@@ -17,6 +17,9 @@
 #ifndef KPERF_MINB
 #define KPERF_MINB 0  // 0: per-app App::MINB
 #endif
+#ifndef KPERF_FOLD
+#define KPERF_FOLD 1  // row scheme: rebuild folded into the vertical pass (fold.cuh)
+#endif
 #ifndef KPERF_MEDCELL
 #define KPERF_MEDCELL 1  // median column NN: cell-grouped lanes + the all-skipped-warp shortcut
 #endif
@@ -590,6 +593,52 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
       }
 #pragma unroll 1
       for (; released < g_end; ++released) mbar_arrive_u32(empty_u32 + 8 * (released & nmask));
+      return;
+    }
+  }
+  // row scheme, fp32, one kept row per period (den 2, or keep-one den 4):
+  // the rebuild folded into the vertical pass (fold.cuh) -- iterate over the
+  // kept rows only: horizontal pass per kept row into a register ring (the
+  // ring slot is released as soon as it is read), then every output row
+  // completed by this kept row as a compile-time weighted sum.  Interior
+  // segments only (no clamped rows); others take the per-row loop below.
+  if constexpr (FAST && SCHEME == S_ROW && sizeof(T) == 4 && App::FOLD && KPERF_FOLD) {
+    const bool interior = ys - VR - m.den >= rp.lim_lo && ye - 1 + VR + m.den <= rp.lim_hi;
+    if (p.fold && interior && (m.den == 2 || (m.den == 4 && m.keep_one))) {
+      auto run = [&](auto dc) {
+        constexpr int DEN = decltype(dc)::value;
+        using F = typename App::template Fold<DEN, RECON>;
+        constexpr int RK = fold_ring(F::sch.span);
+        const int J0 = rp.lo / DEN;  // (rp.lo is a kept row: a multiple of DEN)
+        const float* ringf = reinterpret_cast<const float*>(ring);
+        for (int jb = 0; jb < rp.nload; jb += RK) {
+          static_for<0, RK>([&](auto uc) {
+            constexpr int U = decltype(uc)::value;
+            const int j = jb + U;
+            if (j < rp.nload) {
+              const int gi = g0 + j;
+              mbar_wait_u32(full_u32 + 8 * (gi & nmask), (gi >> p.nr_log2) & 1);
+              const float* row = ringf + (gi & nmask) * slot_elems;
+              const Frag<float, V> c = ldf<float, V>(row + ccol);
+              const Frag<float, EW> el = ldf<float, EW>(row + ecol);
+              const Frag<float, EW> eb = Frag<float, EW>::splat(emode == 1 ? c.get(0) : c.get(V - 1));
+              app.template fold_h<U>(c, emode == 0 ? el : eb, lane, hf);
+              mbar_arrive_u32(empty_u32 + 8 * (gi & nmask));  // the raw row is done with: release its slot
+              const int J = J0 + j;
+              static_for<0, DEN>([&](auto kc) {
+                constexpr int PH = F::sch.order[decltype(kc)::value];
+                const int q = (J - F::sch.tmax[PH]) * DEN + PH;
+                app.template fold_emit<F, RK, U, PH>(q, ys, ye, lane, xc, p, [&](const Frag<float, V>& o) {
+                  store(optr, o);
+                  optr += p.W;
+                });
+              });
+            }
+          });
+        }
+      };
+      if (m.den == 2) run(IC<2>{});
+      else run(IC<4>{});
       return;
     }
   }

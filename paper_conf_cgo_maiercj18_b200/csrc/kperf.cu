@@ -81,7 +81,7 @@ struct perf_plan_s {
   perf_rate rate;
   long long batch = 1, iters = 1, granule_bytes = 128, global_h = -1, band_y0 = 0, tile_w = kp::kNCW, tile_h = 0,
             metric = 0, loader = 0, ring = 0, tile1_w = 16, tile1_h = 16, producer = 0, tblock = 1, p2p = 0,
-            overlap = 1, graph = 1, exchange = 1;
+            overlap = 1, graph = 1, exchange = 1, fold = 1;
   unsigned long long gen = 0;  // bumped by every perf_plan_set (graph keys)
   double* d_err = nullptr;
   float* d_tmp = nullptr;
@@ -228,6 +228,7 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   k.G = G < 1 ? 1 : G;
   const bool rowwise = scheme == PERF_SCHEME_NONE || scheme == PERF_SCHEME_ROW || s1;  // whole rows kept
   k.fast_ok = (rowwise || (k.G % V) == 0) ? 1 : 0;
+  k.fold = (int)P->fold;
   // median, column NN: cells of >= 2 lanes that tile the strip and a warp (kernel.cuh MEDC)
   k.cellmap = (P->app == PERF_APP_MEDIAN && scheme == PERF_SCHEME_COL && P->recon == PERF_RECON_NN && k.den > 1 &&
                k.G % (2 * V) == 0 && k.G <= 32 * V && TW % k.G == 0) ? 1 : 0;
@@ -560,6 +561,10 @@ perf_status perf_plan_set(perf_plan_t p, int key, long long v) {
       if (v < 0 || v > 1) return fail(PERF_ERR_INVALID_ARG, "EXCHANGE must be 0 or 1");
       p->exchange = v;
       return PERF_OK;
+    case PERF_KEY_FOLD:
+      if (v < 0 || v > 1) return fail(PERF_ERR_INVALID_ARG, "FOLD must be 0 or 1");
+      p->fold = v;
+      return PERF_OK;
   }
   return fail(PERF_ERR_INVALID_ARG, "unknown key");
 }
@@ -586,6 +591,7 @@ perf_status perf_plan_get(perf_plan_t p, int key, long long* v) {
     case PERF_KEY_OVERLAP: *v = p->overlap; return PERF_OK;
     case PERF_KEY_GRAPH: *v = p->graph; return PERF_OK;
     case PERF_KEY_EXCHANGE: *v = p->exchange; return PERF_OK;
+    case PERF_KEY_FOLD: *v = p->fold; return PERF_OK;
     case PERF_KEY_CHK_COMPACT: {  // the launch geometry perf_run would use on 256-B aligned buffers
       KParams k;
       unsigned grid;

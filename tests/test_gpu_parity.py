@@ -717,3 +717,23 @@ def test_tma_cell_loads_in_row_bands():
                 kp.perf_run_band(p.handle, buf, out)
                 torch.cuda.synchronize()
             assert torch.equal(out, whole[:, y0:y0 + h]), (scheme, k)
+
+
+@pytest.mark.parametrize("app,r", [("gaussian", 2), ("gaussian", 1), ("sobel", 1), ("sobel", 2), ("gauss_sobel", 2)])
+@pytest.mark.parametrize("rate", [(1, 2), (3, 4)])
+@pytest.mark.parametrize("recon", ["nn", "li"])
+def test_folded_row_rebuild(app, r, rate, recon):
+    """The row scheme's rebuild folded into the vertical pass (fold.cuh,
+    PERF_KEY_FOLD, default on for interior segments): bit-identical to the
+    per-row rebuild-then-filter path (PERF_KEY_FOLD 0) on integer-valued
+    images, and == the oracle.  2 frames of 2048 x 600: 5 row segments per
+    frame, the first and last (image borders) on the per-row path; a ragged
+    tile_h run and a banded run too."""
+    W, H, B = 2048, 600, 2
+    imgs = np.stack([synth.image("natural", 0x5EED2800 + b, W, H) for b in range(B)])
+    fold = gpu_run(app, r, imgs, "row", rate, recon, batch=B)
+    plain = gpu_run(app, r, imgs, "row", rate, recon, batch=B, fold=0)
+    assert np.array_equal(fold, plain)
+    assert np.array_equal(gpu_run(app, r, imgs, "row", rate, recon, batch=B, tile_h=37), plain)
+    want = oracle.run(oracle.params(app, W, H, r, "row", rate, recon), imgs[1])
+    assert_close(app, r, fold[1], want)
