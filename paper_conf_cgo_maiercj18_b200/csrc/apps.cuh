@@ -377,10 +377,12 @@ struct AppGaussSobel {
     else { t[0] = c.v[V - 2]; t[1] = c.v[V - 1]; t[2] = e.v[0]; t[3] = e.v[1]; t[4] = e.v[2]; }
     fke[S] = smooth<2>(t);
   }
-  // Gaussian row q (ys - 1 <= q <= ye); Sobel output row q - 1 once q - 1 >= ys
+  // Gaussian row q; Sobel output row q - 1 stored when ys <= q - 1 < ye.  The
+  // rings advance on every emission, in range or not (values outside the
+  // segment are never stored): no range branch around the ring updates, so no
+  // predicated copies of the ring at the join
   template <class F, int RK, int U, int PH, class Store>
   __device__ __forceinline__ void fold_emit(int q, int ys, int ye, int lane, int xc, const KParams& p, Store&& st) {
-    if (q < ys - 1 || q > ye) return;
     constexpr int SQ = PH % 2, SM = (PH + 1) % 2;  // Sobel ring slots of rows q (and q - 2), q - 1 (DEN even)
     float g[V + 2];
 #pragma unroll
@@ -412,7 +414,7 @@ struct AppGaussSobel {
       o.v[2 * j] = sqrt_approx(m0);
       o.v[2 * j + 1] = sqrt_approx(m1);
     }
-    if (q >= ys + 1) st(o);
+    if (q >= ys + 1 && q <= ye) st(o);
   }
   __device__ void init(const KParams&) {
 #pragma unroll

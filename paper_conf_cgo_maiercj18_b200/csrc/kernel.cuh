@@ -637,9 +637,13 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
           });
         }
       };
+#ifdef KPERF_FOLD_ONLY2  // experiment: one fold instantiation per kernel (instruction-cache footprint)
+      if (m.den == 2) { run(IC<2>{}); return; }
+#else
       if (m.den == 2) run(IC<2>{});
       else run(IC<4>{});
       return;
+#endif
     }
   }
 #if KPERF_PIPELINE
