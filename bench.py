@@ -566,12 +566,24 @@ def main():
         if ws > 1 and args.config == "C2":  # the paths that really exchange data between GPUs
             del x, y, yex
             torch.cuda.empty_cache()
+            # watchdog: the headline line above is complete; if a row-band leg stalls (an NCCL
+            # transport problem on some box), print it with the legs marked and leave
+            def _timeout():
+                for key in ("c4_row_bands", "c2_row_bands"):
+                    result.setdefault(key, {"error": "timeout (watchdog, 300 s)"})
+                if rank == 0:
+                    print(json.dumps(result), flush=True)
+                os._exit(0)
+            wd = threading.Timer(float(os.environ.get("KPERF_BENCH_LEG_TIMEOUT", "300")), _timeout)
+            wd.daemon = True
+            wd.start()
             for key, fn in (("c4_row_bands", lambda: bench_c4_banded(kp, ws, rank, stream)),
                             ("c2_row_bands", lambda: bench_c2_row_bands(kp, ws, rank, stream, args.steps))):
                 try:
                     result[key] = fn()
                 except Exception as e:  # (e.g. NCCL refusing two ranks on one GPU under the gloo test mode)
                     result[key] = {"error": f"{type(e).__name__}: {e}"}
+            wd.cancel()
     if rank == 0 and not args.no_cpu:
         result["cpu_baseline"] = cpu_baseline(cfg)
     if rank == 0:
