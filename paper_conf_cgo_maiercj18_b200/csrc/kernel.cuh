@@ -17,6 +17,9 @@
 #ifndef KPERF_MINB
 #define KPERF_MINB 0  // 0: per-app App::MINB
 #endif
+#ifndef KPERF_SEG_K1
+#define KPERF_SEG_K1 64  // fixed segment height of keep-one row schemes with den >= 4 (see launch_one)
+#endif
 #ifndef KPERF_FOLD
 #define KPERF_FOLD 1  // row scheme: rebuild folded into the vertical pass (fold.cuh)
 #endif
@@ -807,12 +810,15 @@ cudaError_t launch_one(const KParams& p, unsigned grid, size_t smem, cudaStream_
   // (only when that gives >= 2 CTAs per SM: short launches -- perf_run_host's
   // row chunks -- take the wave-filling choice)
   const int n_sms = dev_sms();
+  // keep-one row schemes of den >= 4 re-read up to den - 1 extra kept rows per
+  // segment boundary (halo + rebuild apron): KPERF_SEG_K1-row segments for them
+  const int fseg = (SCHEME == S_ROW && p.keep_one && p.den >= 4) ? KPERF_SEG_K1 : 64;
   const bool fixed64 = p.seg_auto && p.loader == L_BULK && App::VR <= 2 && App::NIN == 1 && sizeof(typename App::T) == 4 &&
-                       SCHEME != S_STENCIL1 &&
-                       (long long)p.n_strips * ((p.y_end - p.y_begin + 63) / 64) * p.frames >= 2LL * n_sms;
+                       SCHEME != S_STENCIL1 && fseg <= p.nrec - 2 * kMaxVR &&
+                       (long long)p.n_strips * ((p.y_end - p.y_begin + fseg - 1) / fseg) * p.frames >= 2LL * n_sms;
   if (fixed64) {
-    q.seg_h = 64;
-    q.n_segs = (p.y_end - p.y_begin + 63) / 64;
+    q.seg_h = fseg;
+    q.n_segs = (p.y_end - p.y_begin + fseg - 1) / fseg;
     grid = (unsigned)((long long)q.n_strips * q.n_segs * q.frames);
   } else if (p.seg_auto) {
     static int per_sm_c[kMaxDev] = {};
