@@ -23,6 +23,9 @@
 #ifndef KPERF_GS_ULI
 #define KPERF_GS_ULI 1
 #endif
+#ifndef KPERF_GS_MINB
+#define KPERF_GS_MINB 3  // fused pipeline: CTAs per SM the registers are budgeted for
+#endif
 
 namespace kp {
 
@@ -348,7 +351,7 @@ struct AppGaussSobel {
   using T = float;
   static constexpr bool ULI = KPERF_GS_ULI;  // uniform row LI (engine.cuh rebuild_frag)
   static constexpr bool IPROD = false;  // PERF_KEY_PRODUCER 2 ignored: a smaller consumer loop (I-cache)
-  static constexpr int V = 8, EW = 4, VR = 3, NIN = 1, NWIN = 4, MINB = 3;
+  static constexpr int V = 8, EW = 4, VR = 3, NIN = 1, NWIN = 4, MINB = KPERF_GS_MINB;
   f2 acc[4][V / 2];  // Gaussian rows in flight (x 256), lane columns, pairs; slot q % 4
   float acce[4];     // the same for the lane's edge column (xc - 1 / xc + V)
   f2 sr[2][V / 2], dr[2][V / 2];  // Sobel horizontal smoothing / derivative of Gaussian rows, slot q % 2
