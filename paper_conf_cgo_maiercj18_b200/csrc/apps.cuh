@@ -23,6 +23,12 @@
 #ifndef KPERF_GS_ULI
 #define KPERF_GS_ULI 1
 #endif
+#ifndef KPERF_FOLD_EDGE
+#define KPERF_FOLD_EDGE 1  // Gaussian / Sobel: the frame's first / last segments fold too (kernel.cuh)
+#endif
+#ifndef KPERF_GS_FOLD_ROT
+#define KPERF_GS_FOLD_ROT 1  // folded C5 loop: one kept row per iteration, register ring shifted (I-cache)
+#endif
 #ifndef KPERF_GS_MINB
 #define KPERF_GS_MINB 3  // fused pipeline: CTAs per SM the registers are budgeted for
 #endif
@@ -141,7 +147,7 @@ struct AppGauss {  // K1 Gaussian, binomial (2R+1)^2, fp32
   f2 h[NWIN][V / 2];  // horizontal results, column pairs (FADD2/FFMA2 vertical pass)
   __device__ void init(const KParams&) {}
   // folded row scheme (fold.cuh): vertical binomial taps incl. the 1/16, 1/256 scale
-  static constexpr bool FOLD = true;
+  static constexpr bool FOLD = true, FOLD_ROT = false, FOLD_EDGE = KPERF_FOLD_EDGE;
   template <int DEN, int RECON>
   struct Fold {
     static constexpr FoldTab tab = fold_tab<DEN, RECON>(BinomTaps<R>::g);
@@ -198,7 +204,7 @@ struct AppSobel {  // K5 Sobel, |(Gx, Gy)|, fp32
   f2 sx[NWIN][V / 2], dx[NWIN][V / 2];  // horizontal smoothing / derivative, column pairs
   __device__ void init(const KParams&) {}
   // folded row scheme (fold.cuh): gx = vertical smoothing of dx, gy = vertical derivative of sx
-  static constexpr bool FOLD = true;
+  static constexpr bool FOLD = true, FOLD_ROT = false, FOLD_EDGE = KPERF_FOLD_EDGE;
   template <int DEN, int RECON>
   struct Fold {
     static constexpr FoldTab tx = fold_tab<DEN, RECON>(BinomTaps<R>::v);
@@ -274,7 +280,7 @@ struct AppInversion {  // K2 Inversion, 255 - x
   static constexpr bool ULI = KPERF_ULI;
   static constexpr bool IPROD = KPERF_IPROD;
   static constexpr int V = 8, EW = 2, VR = 0, NIN = 1, NWIN = 1, MINB = 4;
-  static constexpr bool FOLD = false;
+  static constexpr bool FOLD = false, FOLD_ROT = false, FOLD_EDGE = false;
   __device__ void init(const KParams&) {}
   template <int U>
   __device__ __forceinline__ Frag<float, V> row(const Frag<float, V>& c, const Frag<float, EW>&,
@@ -293,7 +299,7 @@ struct AppHotspot {
   static constexpr bool ULI = KPERF_ULI;
   static constexpr bool IPROD = KPERF_IPROD;
   static constexpr int V = 8, EW = 2, VR = 1, NIN = 2, NWIN = 3, MINB = 4;
-  static constexpr bool FOLD = false;
+  static constexpr bool FOLD = false, FOLD_ROT = false, FOLD_EDGE = false;
   float tc[3][V], tl[3], tr[3], pc[3][V];
   float sdc, rx1, ry1, rz1, amb;
   __device__ void init(const KParams& p) {
@@ -359,7 +365,10 @@ struct AppGaussSobel {
   // results (the Gaussian taps over rebuilt rows folded into kept-row weights);
   // the Sobel stage then runs on every Gaussian row as above (interior rows:
   // no top / bottom clamp)
-  static constexpr bool FOLD = true;
+  // (FOLD_EDGE off: the Sobel stage's clamp in the Gaussian image at the frame's
+  // first / last row would cost a branch per folded emission; those two
+  // segments per frame take the per-row loop and are dispatched first, kernel.cuh)
+  static constexpr bool FOLD = true, FOLD_ROT = KPERF_GS_FOLD_ROT, FOLD_EDGE = false;
   template <int DEN, int RECON>
   struct Fold {
     static constexpr FoldTab tab = fold_tab<DEN, RECON>(BinomTaps<2>::g);
@@ -369,6 +378,8 @@ struct AppGaussSobel {
   };
   f2 fk[8][V / 2];  // kept rows' horizontal Gaussian, ring
   float fke[8];     // ... of the lane's edge column
+  f2 gr[2][V / 2];  // folded loop: Gaussian rows q - 2, q - 1 (slot q % 2), lane columns
+  float grh[2][2];  // ... and their halo columns xc - 1, xc + V
   template <int S>
   __device__ __forceinline__ void fold_h(const Frag<float, V>& c, const Frag<float, EW>& e, int lane, uint32_t) {
     float x[V + 4];
@@ -380,13 +391,22 @@ struct AppGaussSobel {
     else { t[0] = c.v[V - 2]; t[1] = c.v[V - 1]; t[2] = e.v[0]; t[3] = e.v[1]; t[4] = e.v[2]; }
     fke[S] = smooth<2>(t);
   }
+  template <int RK>
+  __device__ __forceinline__ void fold_rotate() {  // FOLD_ROT: kept row k + 1 -> ring position k
+#pragma unroll
+    for (int k = 0; k + 1 < RK; ++k) {
+      fke[k] = fke[k + 1];
+#pragma unroll
+      for (int j = 0; j < V / 2; ++j) fk[k][j] = fk[k + 1][j];
+    }
+  }
   // Gaussian row q; Sobel output row q - 1 stored when ys <= q - 1 < ye.  The
   // rings advance on every emission, in range or not (values outside the
   // segment are never stored): no range branch around the ring updates, so no
   // predicated copies of the ring at the join
   template <class F, int RK, int U, int PH, class Store>
   __device__ __forceinline__ void fold_emit(int q, int ys, int ye, int lane, int xc, const KParams& p, Store&& st) {
-    constexpr int SQ = PH % 2, SM = (PH + 1) % 2;  // Sobel ring slots of rows q (and q - 2), q - 1 (DEN even)
+    constexpr int SQ = PH % 2, SM = (PH + 1) % 2;  // ring slots of Gaussian rows q - 2 (then q), q - 1 (DEN even)
     float g[V + 2];
 #pragma unroll
     for (int j = 0; j < V / 2; ++j)
@@ -404,14 +424,33 @@ struct AppGaussSobel {
 #pragma unroll
       for (int k = 1; k < V + 2; ++k) g[k] = k > cl + 1 ? g[k - 1] : g[k];
     }
+    // vertical first on the Gaussian rows (linear until the magnitude):
+    // S = G(q-2) + 2 G(q-1) + G(q), D = G(q) - G(q-2) on columns -1 .. V;
+    // gx = horizontal derivative of S, gy = horizontal smoothing of D.  The
+    // ring holds Gaussian rows (V + 2 values) instead of the smoothing and
+    // derivative rows (2 V): 12 fewer live registers in the folded loop
+    // (interior segments only: no clamp of the Sobel stage, FOLD_EDGE off)
+    float S[V + 2], D[V + 2];
+#pragma unroll
+    for (int j = 0; j < V / 2; ++j) {
+      const f2 gp = pk2(g[2 * j + 1], g[2 * j + 2]);
+      up2(fma2(splat2(2.f), gr[SM][j], add2(gr[SQ][j], gp)), S[2 * j + 1], S[2 * j + 2]);
+      up2(sub2(gp, gr[SQ][j]), D[2 * j + 1], D[2 * j + 2]);
+    }
+#pragma unroll
+    for (int h = 0; h < 2; ++h) {
+      const int k = h ? V + 1 : 0;
+      S[k] = fmaf(2.f, grh[SM][h], grh[SQ][h] + g[k]);
+      D[k] = g[k] - grh[SQ][h];
+    }
+#pragma unroll
+    for (int j = 0; j < V / 2; ++j) gr[SQ][j] = pk2(g[2 * j + 1], g[2 * j + 2]);
+    grh[SQ][0] = g[0];
+    grh[SQ][1] = g[V + 1];
     Frag<float, V> o;
 #pragma unroll
     for (int j = 0; j < V / 2; ++j) {
-      const f2 sq = smooth_pair<1>(g + 2 * j), dq = deriv_pair<1>(g + 2 * j);
-      const f2 gx = fma2(splat2(2.f), dr[SM][j], add2(dr[SQ][j], dq));
-      const f2 gy = sub2(sq, sr[SQ][j]);
-      sr[SQ][j] = sq;
-      dr[SQ][j] = dq;
+      const f2 gx = deriv_pair<1>(S + 2 * j), gy = smooth_pair<1>(D + 2 * j);
       float m0, m1;
       up2(fma2(gx, gx, mul2(gy, gy)), m0, m1);
       o.v[2 * j] = sqrt_approx(m0);
@@ -427,9 +466,11 @@ struct AppGaussSobel {
       for (int j = 0; j < V / 2; ++j) acc[k][j] = splat2(0.f);
     }
 #pragma unroll
-    for (int k = 0; k < 2; ++k)
+    for (int k = 0; k < 2; ++k) {
 #pragma unroll
-      for (int j = 0; j < V / 2; ++j) sr[k][j] = dr[k][j] = splat2(0.f);
+      for (int j = 0; j < V / 2; ++j) sr[k][j] = dr[k][j] = gr[k][j] = splat2(0.f);
+      grh[k][0] = grh[k][1] = 0.f;
+    }
   }
   template <int U>
   __device__ __forceinline__ Frag<float, V> row(const Frag<float, V>& c, const Frag<float, EW>& e,
@@ -477,20 +518,39 @@ struct AppGaussSobel {
       for (int k = 1; k < V + 2; ++k) g[k] = k > cl + 1 ? g[k - 1] : g[k];
     }
     // Sobel3 on Gaussian rows oy-1, oy, oy+1 (oy = vy - 3 = gy - 1); clamp coefficients (warp uniform)
+    // (rows away from the image's first / last row -- all but two per frame --
+    // take the plain form: a warp-uniform branch, no per-row coefficient work)
     const int oy = vy - 3;
-    const float top = oy == 0 ? 1.f : 0.f, bot = oy == p.Hg - 1 ? 1.f : 0.f;
-    const f2 kt = splat2(1.f - top), kb = splat2(1.f - bot), km = splat2(2.f + top + bot);
-    const f2 kst = splat2(top - 1.f), ksm = splat2(bot - top);
+    const bool edge = oy <= 0 || oy >= p.Hg - 1;
+    f2 sq[V / 2], dq[V / 2], gx[V / 2], gy[V / 2];
+#pragma unroll
+    for (int j = 0; j < V / 2; ++j) {
+      sq[j] = smooth_pair<1>(g + 2 * j);
+      dq[j] = deriv_pair<1>(g + 2 * j);
+    }
+    if (!edge) {
+#pragma unroll
+      for (int j = 0; j < V / 2; ++j) {
+        gx[j] = fma2(splat2(2.f), dr[SM][j], add2(dr[SQ][j], dq[j]));
+        gy[j] = sub2(sq[j], sr[SQ][j]);
+      }
+    } else {
+      const float top = oy == 0 ? 1.f : 0.f, bot = oy == p.Hg - 1 ? 1.f : 0.f;
+      const f2 kt = splat2(1.f - top), kb = splat2(1.f - bot), km = splat2(2.f + top + bot);
+      const f2 kst = splat2(top - 1.f), ksm = splat2(bot - top);
+#pragma unroll
+      for (int j = 0; j < V / 2; ++j) {
+        gx[j] = fma2(km, dr[SM][j], fma2(kt, dr[SQ][j], mul2(kb, dq[j])));
+        gy[j] = fma2(kb, sq[j], fma2(ksm, sr[SM][j], mul2(kst, sr[SQ][j])));
+      }
+    }
     Frag<float, V> o;
 #pragma unroll
     for (int j = 0; j < V / 2; ++j) {
-      const f2 sq = smooth_pair<1>(g + 2 * j), dq = deriv_pair<1>(g + 2 * j);
-      const f2 gx = fma2(km, dr[SM][j], fma2(kt, dr[SQ][j], mul2(kb, dq)));
-      const f2 gy = fma2(kb, sq, fma2(ksm, sr[SM][j], mul2(kst, sr[SQ][j])));
-      sr[SQ][j] = sq;
-      dr[SQ][j] = dq;
+      sr[SQ][j] = sq[j];
+      dr[SQ][j] = dq[j];
       float m0, m1;
-      up2(fma2(gx, gx, mul2(gy, gy)), m0, m1);
+      up2(fma2(gx[j], gx[j], mul2(gy[j], gy[j])), m0, m1);
       o.v[2 * j] = sqrt_approx(m0);
       o.v[2 * j + 1] = sqrt_approx(m1);
     }
@@ -527,7 +587,7 @@ struct AppMedian {
   // (kernel.cuh MEDC) leave the kept warps as the critical path; more resident
   // CTAs hide their latency (C3 col 1/2 NN 235 -> 196 us, exact 230 -> 228 us)
   static constexpr int V = 16, EW = 4, VR = 1, NIN = 1, NWIN = 3, MINB = 4;
-  static constexpr bool FOLD = false;
+  static constexpr bool FOLD = false, FOLD_ROT = false, FOLD_EDGE = false;
   static constexpr int NW = V / 2 + 2;  // 16-bit-pair words per row incl. the two halo words
   uint32_t r[3][NW];  // word 0 = (_, col -1), words 1..V/2 = cols 0..V-1, last = (col V, _)
   __device__ void init(const KParams&) {}

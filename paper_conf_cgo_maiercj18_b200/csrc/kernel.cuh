@@ -23,6 +23,9 @@
 #ifndef KPERF_FOLD
 #define KPERF_FOLD 1  // row scheme: rebuild folded into the vertical pass (fold.cuh)
 #endif
+#ifndef KPERF_LPT
+#define KPERF_LPT 1  // folded row scheme: a frame's first / last segments dispatched first
+#endif
 #ifndef KPERF_MEDCELL
 #define KPERF_MEDCELL 1  // median column NN: cell-grouped lanes + the all-skipped-warp shortcut
 #endif
@@ -30,6 +33,12 @@
 namespace kp {
 
 constexpr int kMaxVR = 3;  // largest vertical radius of an app (recipe table rows = seg_h + 2 VR)
+// recipe-table padding: the unrolled row loops run whole groups of NWIN rows
+// (NWIN <= 5); rows past the segment's last virtual row repeat its recipe with
+// emit = 0 (no ring wait or release, no store), so the unrolled body has no
+// per-row guard -- a guard is a join point where every register-ring value
+// needs a copy (C5 exact: 260 -> 220 SASS instructions per row)
+constexpr int kRecPad = 8;
 
 // per-device host caches (a process may drive several devices through one
 // library: kernel attributes, SM counts and occupancy are per device)
@@ -566,8 +575,8 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
       for (int ib = 0; ib < nv; ib += 3) {
         auto unrolled = [&](auto uc) {
           constexpr int U = decltype(uc)::value, A = (U + 1) % 3, B = (U + 2) % 3;
-          const int i = ib + U;
-          if (i < nv) {
+          const int i = ib + U;  // (rows >= nv: padded recipes -- no wait, no store)
+          {
             const Recipe rec = sync(i, true);
             const T* row = ring_at(ring, rec.oa);
             abw[U] = (uint32_t)row[ca] | ((uint32_t)row[cb] << 16);
@@ -606,28 +615,61 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
   // completed by this kept row as a compile-time weighted sum.  Interior
   // segments only (no clamped rows); others take the per-row loop below.
   if constexpr (FAST && SCHEME == S_ROW && sizeof(T) == 4 && App::FOLD && KPERF_FOLD) {
-    const bool interior = ys - VR - m.den >= rp.lim_lo && ye - 1 + VR + m.den <= rp.lim_hi;
-    if (p.fold && interior && (m.den == 2 || (m.den == 4 && m.keep_one))) {
+    // Segments at the image's top / bottom row fold too: the clamp-to-edge
+    // rebuilt image (R8) equals the kept-row lattice extended by copies of
+    // the first / last kept row (LI between two equal rows, NN of equal rows:
+    // the copy), so arrivals above the first and below the last loaded row
+    // re-read those rows' slots ("virtual arrivals").  Buffer limits that are
+    // not image rows (band halos) still need the margin.
+    const bool top_ok = ys - VR - m.den >= rp.lim_lo || (App::FOLD_EDGE && p.avail0 <= 0);
+    const bool bot_ok = ye - 1 + VR + m.den <= rp.lim_hi || (App::FOLD_EDGE && p.avail1 >= p.Hg);
+    if (p.fold && top_ok && bot_ok && (m.den == 2 || (m.den == 4 && m.keep_one))) {
       auto run = [&](auto dc) {
         constexpr int DEN = decltype(dc)::value;
         using F = typename App::template Fold<DEN, RECON>;
         constexpr int RK = fold_ring(F::sch.span);
-        const int J0 = rp.lo / DEN;  // (rp.lo is a kept row: a multiple of DEN)
+        // FOLD_ROT: one arrival per loop iteration, the newest kept row at ring
+        // position RK - 1 and the ring shifted down after its emissions (RK - 1
+        // register moves) -- a quarter of the unrolled code (instruction cache)
+        constexpr int UN = App::FOLD_ROT ? 1 : RK;
+        const int J0 = rp.lo / DEN;  // first loaded kept row (rp.lo is a multiple of DEN)
+        auto fdiv = [](int a) { return a >= 0 ? a / DEN : -((-a + DEN - 1) / DEN); };
+        // kept rows the segment's outputs read: the loaded ones, plus (FOLD_EDGE,
+        // image border segments) virtual arrivals of the first / last loaded row
+        const int Js = App::FOLD_EDGE ? fdiv(ys - VR) : J0;
+        const int Je = App::FOLD_EDGE ? -fdiv(-(ye - 1 + VR)) : J0 + rp.nload - 1;
+        const int na = Je - Js + 1;
         const float* ringf = reinterpret_cast<const float*>(ring);
-        for (int jb = 0; jb < rp.nload; jb += RK) {
-          static_for<0, RK>([&](auto uc) {
-            constexpr int U = decltype(uc)::value;
-            const int j = jb + U;
-            if (j < rp.nload) {
-              const int gi = g0 + j;
-              mbar_wait_u32(full_u32 + 8 * (gi & nmask), (gi >> p.nr_log2) & 1);
+#pragma unroll 1
+        for (int jb = 0; jb < na; jb += UN) {
+          static_for<0, UN>([&](auto uc) {
+            constexpr int U = App::FOLD_ROT ? RK - 1 : decltype(uc)::value;  // ring position of this arrival
+            // (arrivals past the last one, J > Je, only occur in the last unrolled
+            // group of the non-rotating ring: skipped -- measured: the guard keeps
+            // the Gaussian / Sobel fold loops free of spills)
+            const int J = Js + jb + (App::FOLD_ROT ? 0 : U);
+            int gi;
+            bool wait, release;
+            if constexpr (App::FOLD_EDGE) {
+              const int r = J - J0;  // loaded-row index (< 0 / >= nload: virtual, the first / last row's slot)
+              gi = g0 + min(max(r, 0), rp.nload - 1);
+              wait = J <= Je && r < rp.nload;
+              release = J <= Je && r >= 0 && r < rp.nload;
+            } else {
+              gi = g0 + (J - J0);
+              wait = release = J <= Je;
+            }
+            if (App::FOLD_ROT || J <= Je) {
+              if (wait) mbar_wait_u32(full_u32 + 8 * (gi & nmask), (gi >> p.nr_log2) & 1);
               const float* row = ringf + (gi & nmask) * slot_elems;
               const Frag<float, V> c = ldf<float, V>(row + ccol);
               const Frag<float, EW> el = ldf<float, EW>(row + ecol);
               const Frag<float, EW> eb = Frag<float, EW>::splat(emode == 1 ? c.get(0) : c.get(V - 1));
               app.template fold_h<U>(c, emode == 0 ? el : eb, lane, hf);
-              mbar_arrive_u32(empty_u32 + 8 * (gi & nmask));  // the raw row is done with: release its slot
-              const int J = J0 + j;
+              // the raw row is done with: release its slot (virtual arrivals of the
+              // first row precede its own; those of the last row follow it -- no
+              // further loads, so its slot keeps its data)
+              if (release) mbar_arrive_u32(empty_u32 + 8 * (gi & nmask));
               static_for<0, DEN>([&](auto kc) {
                 constexpr int PH = F::sch.order[decltype(kc)::value];
                 const int q = (J - F::sch.tmax[PH]) * DEN + PH;
@@ -638,6 +680,7 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
               });
             }
           });
+          if constexpr (App::FOLD_ROT) app.template fold_rotate<RK>();
         }
       };
 #ifdef KPERF_FOLD_ONLY2  // experiment: one fold instantiation per kernel (instruction-cache footprint)
@@ -668,7 +711,7 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
   for (int ib = 0; ib < nv; ib += NWIN) {
     auto unrolled = [&](auto uc) {
       const int i = ib + decltype(uc)::value;
-      if (i < nv) compute(uc, fetch(i), vy0 + i);  // (vy only matters to the fused Gauss-Sobel)
+      compute(uc, fetch(i), vy0 + i);  // (rows >= nv: padded recipes, emit 0; vy only matters to the fused Gauss-Sobel)
     };
     static_for<0, NWIN>(unrolled);
   }
@@ -748,10 +791,30 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : (NCW
     const int item = blockIdx.x;  // one work item per CTA (persistent variant)
     if (item >= n_items) return;
     int b = item;
-    const int strip = b % p.n_strips;
-    b /= p.n_strips;
-    const int seg = b % p.n_segs;
-    const int frame = b / p.n_segs;
+    int strip, seg, frame;
+    // folded row scheme without FOLD_EDGE: the first and last segment of a frame take the
+    // per-row loop (clamped rows) and run ~1.5x longer than the folded
+    // interior ones -- dispatch them first (longest items first), so they do
+    // not form the launch's tail (C5: SMs idle 19% of the kernel otherwise)
+    constexpr bool LPT = KPERF_LPT && SCHEME == S_ROW && App::FOLD && !App::FOLD_EDGE && KPERF_FOLD && sizeof(T) == 4;
+    if (LPT && p.fold && p.n_segs >= 3 && (m.den == 2 || (m.den == 4 && m.keep_one)) &&
+        b < 2 * p.n_strips * p.frames) {
+      strip = b % p.n_strips;
+      b /= p.n_strips;
+      seg = (b & 1) ? p.n_segs - 1 : 0;
+      frame = b >> 1;
+    } else if (LPT && p.fold && p.n_segs >= 3 && (m.den == 2 || (m.den == 4 && m.keep_one))) {
+      b -= 2 * p.n_strips * p.frames;
+      strip = b % p.n_strips;
+      b /= p.n_strips;
+      seg = 1 + b % (p.n_segs - 2);
+      frame = b / (p.n_segs - 2);
+    } else {
+      strip = b % p.n_strips;
+      b /= p.n_strips;
+      seg = b % p.n_segs;
+      frame = b / p.n_segs;
+    }
     (void)strip;  // (x0 above)
     const int ys = p.y_begin + seg * p.seg_h;
     const int ye = min(ys + p.seg_h, p.y_end);
@@ -761,10 +824,11 @@ __global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : (NCW
     } else {
       const int nv = n_recipes<SCHEME>(p, ys, ye, App::VR);
       __syncwarp();
-      for (int i = lane; i < nv; i += 32) {
+      const int nv_pad = (nv + App::NWIN - 1) / App::NWIN * App::NWIN;  // (<= nv + kRecPad)
+      for (int i = lane; i < nv_pad; i += 32) {
         int emit;
-        const int y = virtual_row<SCHEME>(p, rp, ys, ye, App::VR, i, emit);
-        rtab[i] = make_recipe<SCHEME, RECON>(p, m, rp, y, emit, slot_elems * (int)sizeof(T));
+        const int y = virtual_row<SCHEME>(p, rp, ys, ye, App::VR, min(i, nv - 1), emit);
+        rtab[i] = make_recipe<SCHEME, RECON>(p, m, rp, y, i < nv ? emit : 0, slot_elems * (int)sizeof(T));
       }
       __syncwarp();
       const int xw = x0 + (warp - cw0) * 32 * V;
@@ -814,7 +878,7 @@ cudaError_t launch_one(const KParams& p, unsigned grid, size_t smem, cudaStream_
   // segment boundary (halo + rebuild apron): KPERF_SEG_K1-row segments for them
   const int fseg = (SCHEME == S_ROW && p.keep_one && p.den >= 4) ? KPERF_SEG_K1 : 64;
   const bool fixed64 = p.seg_auto && p.loader == L_BULK && App::VR <= 2 && App::NIN == 1 && sizeof(typename App::T) == 4 &&
-                       SCHEME != S_STENCIL1 && fseg <= p.nrec - 2 * kMaxVR &&
+                       SCHEME != S_STENCIL1 && fseg <= p.nrec - 2 * kMaxVR - kRecPad &&
                        (long long)p.n_strips * ((p.y_end - p.y_begin + fseg - 1) / fseg) * p.frames >= 2LL * n_sms;
   if (fixed64) {
     q.seg_h = fseg;

@@ -339,7 +339,7 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   int seg = (int)(P->tile_h > 0 ? P->tile_h : (nin == 2 ? 64 : 128));
   if (s1) seg = (seg + k.tile1_h - 1) / k.tile1_h * k.tile1_h;  // whole Stencil1 tiles per segment
   // recipes per segment: seg + 2 VR rows, Stencil1: every tile restarts its window
-  k.nrec = s1 ? seg + (seg / k.tile1_h + 1) * 2 * kp::kMaxVR : seg + 2 * kp::kMaxVR;
+  k.nrec = (s1 ? seg + (seg / k.tile1_h + 1) * 2 * kp::kMaxVR : seg + 2 * kp::kMaxVR) + kp::kRecPad;
   // + the column scheme's per-lane LI weight tables / the checkerboard's phase table
   // (fp32; kernel.cuh ctab: 3 x 32 float4 per consumer warp)
   size_t col_tab = 0;
