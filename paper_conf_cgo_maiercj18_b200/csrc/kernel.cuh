@@ -711,7 +711,10 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
   for (int ib = 0; ib < nv; ib += NWIN) {
     auto unrolled = [&](auto uc) {
       const int i = ib + decltype(uc)::value;
-      compute(uc, fetch(i), vy0 + i);  // (rows >= nv: padded recipes, emit 0; vy only matters to the fused Gauss-Sobel)
+      // (rows >= nv: padded recipes, emit 0; vy only matters to the fused Gauss-Sobel).
+      // The median's column-NN kernel keeps the guard (measured: its kept
+      // warps are the critical path and gain nothing from the copies saved)
+      if (!MEDC || i < nv) compute(uc, fetch(i), vy0 + i);
     };
     static_for<0, NWIN>(unrolled);
   }
