@@ -18,7 +18,10 @@
 #define KPERF_MINB 0  // 0: per-app App::MINB
 #endif
 #ifndef KPERF_SEG_K1
-#define KPERF_SEG_K1 64  // fixed segment height of keep-one row schemes with den >= 4 (see launch_one)
+#define KPERF_SEG_K1 24  // fixed segment height of keep-one row schemes with den >= 4 (see launch_one)
+#endif
+#ifndef KPERF_SEG_FIX
+#define KPERF_SEG_FIX 16  // fixed segment height of the other fp32 whole-row kernels (see launch_one)
 #endif
 #ifndef KPERF_FOLD
 #define KPERF_FOLD 1  // row scheme: rebuild folded into the vertical pass (fold.cuh)
@@ -869,17 +872,23 @@ cudaError_t launch_one(const KParams& p, unsigned grid, size_t smem, cudaStream_
   // (occupancy API), discounted by the per-segment halo rows.
   KParams q = p;
   if (!App::IPROD) q.inline_prod = 0;  // (no inline-producer code in this app's consumer loop)
-  // fp32 whole-row (TMA bulk) loaders, one input, radius <= 2: fixed 64-row
-  // segments -- several waves of short items balance better than the
-  // wave-filling choice below (C2: row 1/2 0.178 -> 0.170 ms, exact 0.193 ->
-  // 0.181 ms; tools/sweep_tile_h.py).  Cell loaders, u8, Hotspot and the
-  // fused pipeline measured best with the wave-filling choice.
+  // fp32 whole-row (TMA bulk) loaders, one input, radius <= 2: short fixed
+  // segments -- many waves of short items overlap one CTA's ring fill and
+  // drain with the others' streaming (round 2b sweep, tools/sweep_ring.py,
+  // profiles/r02/sweep_ring_row.txt: 16-row segments, keep-one den >= 4 24
+  // rows; C2 Gaussian5 exact 178 -> 165 us, row 1/2 LI 137 -> 130 us, row 3/4
+  // 119 -> 110 us -- the extra halo reads of the neighbouring segment hit L2).
+  // Cell loaders, u8, Hotspot and the fused pipeline measured best with the
+  // wave-filling choice.
   // (only when that gives >= 2 CTAs per SM: short launches -- perf_run_host's
   // row chunks -- take the wave-filling choice)
   const int n_sms = dev_sms();
   // keep-one row schemes of den >= 4 re-read up to den - 1 extra kept rows per
   // segment boundary (halo + rebuild apron): KPERF_SEG_K1-row segments for them
-  const int fseg = (SCHEME == S_ROW && p.keep_one && p.den >= 4) ? KPERF_SEG_K1 : 64;
+  // (narrow 2-warp CTAs, C1's 512^2 frames: the row scheme keeps 64-row
+  // segments -- Gaussian5 row 1/2 LI 135.6 us vs 145.6 with 16 rows)
+  const int fseg = (SCHEME == S_ROW && NCW == 2) ? 64
+                   : (SCHEME == S_ROW && p.keep_one && p.den >= 4) ? KPERF_SEG_K1 : KPERF_SEG_FIX;
   const bool fixed64 = p.seg_auto && p.loader == L_BULK && App::VR <= 2 && App::NIN == 1 && sizeof(typename App::T) == 4 &&
                        SCHEME != S_STENCIL1 && fseg <= p.nrec - 2 * kMaxVR - kRecPad &&
                        (long long)p.n_strips * ((p.y_end - p.y_begin + fseg - 1) / fseg) * p.frames >= 2LL * n_sms;

@@ -330,6 +330,14 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   if (scheme == PERF_SCHEME_ROW) hold = 2;
   if (scheme == PERF_SCHEME_CHECKER) hold = 2 * (k.keep_one ? k.den - 1 : 1) + 1;  // rows a cell's rebuild spans
   int nr = P->ring > 0 ? next_pow2((int)P->ring) : next_pow2(hold + (hold > 2 ? 4 : 6));
+  // fp32 column scheme, skip-one 1/4 and NN 1/2: a 4-row ring (the producer at
+  // most 4 rows ahead) measured faster than 8 (C2: Gaussian5 col 1/4 NN 175 ->
+  // 162 us, LI 171 -> 164, Sobel3 col 1/4 NN 175 -> 160, col 1/2 NN 153 ->
+  // 147 us; LI 1/2 and 3/4 are faster with 8: tools/sweep_ring.py,
+  // profiles/r02/sweep_ring_col.txt)
+  if (P->ring == 0 && scheme == PERF_SCHEME_COL && es == 4 && k.den > 1 &&
+      ((k.den == 4 && P->rate.num == 1) || (k.den == 2 && P->recon == PERF_RECON_NN)))
+    nr = 4;
   if (nr < hold + 1) nr = next_pow2(hold + 1);
   const int nin = P->app == PERF_APP_HOTSPOT ? 2 : 1;
   const size_t slot_bytes = (size_t)k.row_elems * nin * es;
