@@ -477,12 +477,14 @@ def main():
         plan = kp.Plan(app, W, H, cfg["r"], cfg["scheme"], cfg["rate"], cfg["recon"], batch=B, granule_bytes=G)
         exact = kp.Plan(app, W, H, cfg["r"], "none", (0, 1), "nn", batch=B)
         run = lambda: plan.run(x, y, stream)  # noqa: E731
-        for _ in range(args.warmup):
-            run()
-        torch.cuda.synchronize()
-        barrier(ws)
-        torch.cuda.synchronize()
+        # (the warm-up runs inside the clock sampler: its start-up pause would
+        # otherwise leave the GPU idle for 0.3 s right before the timed steps)
         with ClockSampler(local) as clk:
+            for _ in range(args.warmup):
+                run()
+            torch.cuda.synchronize()
+            barrier(ws)
+            torch.cuda.synchronize()
             e0 = torch.cuda.Event(enable_timing=True)
             e1 = torch.cuda.Event(enable_timing=True)
             e0.record(stream)
@@ -870,11 +872,11 @@ def bench_hotspot(args, cfg, ws, rank, local, stream, peak, peak_src):
         kp.perf_comm_init(plan.handle, uid, rank, ws)
         kp.perf_comm_init(exact.handle, uid, rank, ws)
     run = lambda: plan.hotspot(T, P, out, stream)  # noqa: E731
-    for _ in range(args.warmup):
-        run()
-    torch.cuda.synchronize()
-    barrier(ws)
-    with ClockSampler(local) as clk:
+    with ClockSampler(local) as clk:  # (warm-up inside: no idle gap before the timed steps)
+        for _ in range(args.warmup):
+            run()
+        torch.cuda.synchronize()
+        barrier(ws)
         e0 = torch.cuda.Event(enable_timing=True)
         e1 = torch.cuda.Event(enable_timing=True)
         e0.record(stream)

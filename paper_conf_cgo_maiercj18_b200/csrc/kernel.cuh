@@ -29,6 +29,9 @@
 #ifndef KPERF_LPT
 #define KPERF_LPT 1  // folded row scheme: a frame's first / last segments dispatched first
 #endif
+#ifndef KPERF_MEDC_ILV
+#define KPERF_MEDC_ILV 1  // median column NN: interleaved warp ranks (C3 col 1/2 NN 197 -> 183 us)
+#endif
 #ifndef KPERF_MEDCELL
 #define KPERF_MEDCELL 1  // median column NN: cell-grouped lanes + the all-skipped-warp shortcut
 #endif
@@ -167,7 +170,10 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
     if (p.cellmap && x0 + TW <= p.W) {
       cellmap = true;
       const int lpc = p.G / V, ncell = TW / p.G, c0 = x0 / p.G;
-      const int want = w * (32 / lpc) + lane / lpc;
+      // warp rank: KPERF_MEDC_ILV interleaves the ranks (0, 2, 1, 3 for four
+      // warps) so the kept-cell warps (ranks first) are not adjacent warp ids
+      const int rank = (KPERF_MEDC_ILV && NCW == 4) ? ((w & 1) << 1 | (w >> 1)) : w;
+      const int want = rank * (32 / lpc) + lane / lpc;
       int nk = 0;
       for (int j = 0; j < ncell; ++j) nk += m.phase_kept((c0 + j) % m.den) ? 1 : 0;
       int cell = 0, kk = 0, ks = 0;
