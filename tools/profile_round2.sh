@@ -34,8 +34,7 @@ for v in all c1 c3all c5; do
 done
 ncu --metrics $M --clock-control none -k regex:perf_kernel --csv --log-file $O/ncu_variants_all_g1px.csv \
   python tools/ncu_driver.py --variants all --batch 2 --gran 4 > $O/ncu_variants_all_g1px.log 2>&1
-# sanitizers
-for t in memcheck racecheck synccheck; do
-  compute-sanitizer --tool $t --print-limit 20 python tests/_sanitizer_workload.py > $O/sanitizer_$t.log 2>&1
-done
+# sanitizers: compute-sanitizer is closed on the GPU pool since round 2b (runs
+# under it left GPUs needing a reset); the committed round-2 logs
+# (profiles/r02/sanitizer_*.log) predate the 2b kernel changes
 ls -la $O
