@@ -630,11 +630,12 @@ def bench_e2e(kp, cfg, stream, args, ws, x):
     e1.record(stream)
     e1.synchronize()
     ms = max_over_ranks(ws, e0.elapsed_time(e1) / steps)
-    plan.close()
     nb = W * H * (1 if u8 else 4)
+    h2d = plan.get("h2d_bytes")  # row scheme: only the kept rows cross PCIe (PERF_KEY_HOST_SKIP)
+    plan.close()
     return {"value": ws * W * H / (ms * 1e-3) / 1e6, "unit": "Mpixel/s" if app != "hotspot" else "Mcell-updates/s",
-            "h2d_bytes_per_step": nb, "d2h_bytes_per_step": nb, "ms_per_step": ms,
-            "api": "perf_run_host (pinned host buffers, one frame per step)"}
+            "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": nb, "ms_per_step": ms,
+            "api": "perf_run_host (pinned host buffers, one frame per step; row scheme: kept rows only host->device)"}
 
 
 def bench_variants(kp, cfg, x, y, yex, stream, peak, ws):

@@ -125,11 +125,16 @@ enum {
                                   Reads 2 after a capture failed and the plan fell back to eager launches */
   PERF_KEY_EXCHANGE = 20,      /* MEASUREMENT ONLY: 0 skips every halo exchange of banded runs (results are
                                   then wrong at band edges) so the exchange's share of a step can be timed */
-  PERF_KEY_FOLD = 21           /* row scheme, fp32 Gaussian / Sobel / Gauss-Sobel, one kept row per period (den 2
+  PERF_KEY_FOLD = 21,          /* row scheme, fp32 Gaussian / Sobel / Gauss-Sobel, one kept row per period (den 2
                                   or keep-one den 4): 1 (default) = the rebuild is folded into the vertical pass
                                   -- per kept row one horizontal pass, each output row a compile-time weighted
                                   sum of kept rows; 0 = rebuild every row,
                                   then filter.  Same values (bit-identical on integer-valued inputs) */
+  PERF_KEY_HOST_SKIP = 22,     /* perf_run_host, row scheme: 1 (default) = only the kept rows are copied host ->
+                                  device (one strided 2-D copy per kept phase; the kernels never read a skipped
+                                  row, so the perforation saves PCIe bytes as well as HBM bytes); 0 = whole
+                                  frames.  Same results */
+  PERF_KEY_H2D_BYTES = 23      /* read-only: bytes one perf_run_host call copies host -> device (BATCH frames) */
 };
 
 /* size of a perf_p2p_export handle */
@@ -156,7 +161,9 @@ perf_status perf_run_host(perf_plan_t plan, const void* host_in, void* host_out,
 /* (Pipelined: the batch is cut into <= 16 row chunks; chunk i is copied in on a
  * plan-owned stream, the output rows it completes are computed on `stream`, and
  * copied out on a second plan-owned stream, so both PCIe directions and the
- * kernels overlap.  Host buffers should be pinned for the copies to overlap.) */
+ * kernels overlap.  Host buffers should be pinned for the copies to overlap.
+ * Row scheme: only the kept rows are copied in (PERF_KEY_HOST_SKIP); the
+ * device staging copy of a skipped row is never read.) */
 
 /* ITERS Hotspot steps on device buffers of W * H floats (a band of H rows
  * starting at global row BAND_Y0 of a GLOBAL_H-row grid when sharded).  T and

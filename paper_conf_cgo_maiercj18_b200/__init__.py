@@ -23,7 +23,8 @@ RECON = {"nn": 0, "li": 1, "linear": 1}
 METRIC = {"mre": 0, "me": 1, "mae": 2}
 KEY = {"batch": 1, "iters": 2, "granule_bytes": 3, "global_h": 4, "band_y0": 5, "tile_w": 6, "tile_h": 7,
        "metric": 8, "loader": 9, "ring": 10, "halo_rows": 11, "tile1_w": 12, "tile1_h": 13, "producer": 14,
-       "tblock": 15, "p2p": 16, "chk_compact": 17, "overlap": 18, "graph": 19, "exchange": 20, "fold": 21}
+       "tblock": 15, "p2p": 16, "chk_compact": 17, "overlap": 18, "graph": 19, "exchange": 20, "fold": 21,
+       "host_skip": 22, "h2d_bytes": 23}
 STATUS = {0: "PERF_OK", 1: "PERF_ERR_INVALID_ARG", 2: "PERF_ERR_UNSUPPORTED", 3: "PERF_ERR_CUDA",
           4: "PERF_ERR_NCCL", 5: "PERF_ERR_OOM"}
 

@@ -81,7 +81,7 @@ struct perf_plan_s {
   perf_rate rate;
   long long batch = 1, iters = 1, granule_bytes = 128, global_h = -1, band_y0 = 0, tile_w = kp::kNCW, tile_h = 0,
             metric = 0, loader = 0, ring = 0, tile1_w = 16, tile1_h = 16, producer = 0, tblock = 1, p2p = 0,
-            overlap = 1, graph = 1, exchange = 1, fold = 1;
+            overlap = 1, graph = 1, exchange = 1, fold = 1, host_skip = 1;
   unsigned long long gen = 0;  // bumped by every perf_plan_set (graph keys)
   double* d_err = nullptr;
   float* d_tmp = nullptr;
@@ -483,6 +483,8 @@ perf_status perf_plan(perf_plan_t* plan, perf_app app, int W, int H, int radius,
 static void host_graph_free(perf_plan_s* p);
 static void hotspot_graph_free(perf_plan_s* p);
 
+static long long host_h2d_bytes(const perf_plan_s* p);  // (perf_run_host section)
+
 perf_status perf_plan_set(perf_plan_t p, int key, long long v) {
   if (!p) return fail(PERF_ERR_INVALID_ARG, "plan is NULL");
   host_graph_free(p);  // a captured perf_run_host pipeline bakes in the plan's launch parameters
@@ -573,6 +575,12 @@ perf_status perf_plan_set(perf_plan_t p, int key, long long v) {
       if (v < 0 || v > 1) return fail(PERF_ERR_INVALID_ARG, "FOLD must be 0 or 1");
       p->fold = v;
       return PERF_OK;
+    case PERF_KEY_HOST_SKIP:
+      if (v < 0 || v > 1) return fail(PERF_ERR_INVALID_ARG, "HOST_SKIP must be 0 or 1");
+      p->host_skip = v;
+      return PERF_OK;
+    case PERF_KEY_H2D_BYTES:
+      return fail(PERF_ERR_INVALID_ARG, "H2D_BYTES is read-only");
   }
   return fail(PERF_ERR_INVALID_ARG, "unknown key");
 }
@@ -600,6 +608,8 @@ perf_status perf_plan_get(perf_plan_t p, int key, long long* v) {
     case PERF_KEY_GRAPH: *v = p->graph; return PERF_OK;
     case PERF_KEY_EXCHANGE: *v = p->exchange; return PERF_OK;
     case PERF_KEY_FOLD: *v = p->fold; return PERF_OK;
+    case PERF_KEY_HOST_SKIP: *v = p->host_skip; return PERF_OK;
+    case PERF_KEY_H2D_BYTES: *v = host_h2d_bytes(p); return PERF_OK;
     case PERF_KEY_CHK_COMPACT: {  // the launch geometry perf_run would use on 256-B aligned buffers
       KParams k;
       unsigned grid;
@@ -669,6 +679,23 @@ static cudaError_t host_pipe_init(perf_plan_s* p) {
   return e;
 }
 
+// perf_run_host, row scheme (HOST_SKIP): which rows cross PCIe
+static bool host_row_skip(const perf_plan_s* p) {
+  return p->host_skip && p->scheme == PERF_SCHEME_ROW && p->rate.num > 0 && p->rate.den > 1;
+}
+static bool host_phase_kept(const perf_plan_s* p, int ph) {  // (R2: phase 0 always kept; keep-one keeps phase 0 only)
+  return p->rate.num == p->rate.den - 1 ? ph == 0 : ph != p->rate.den - 1;
+}
+static long long host_h2d_bytes(const perf_plan_s* p) {  // bytes perf_run_host copies in per call
+  const long long row = (long long)p->W * (long long)elem_size(p->app);
+  long long rows = p->H;
+  if (host_row_skip(p)) {
+    rows = 0;
+    for (int y = 0; y < p->H; ++y) rows += host_phase_kept(p, y % p->rate.den) ? 1 : 0;
+  }
+  return rows * row * p->batch;
+}
+
 // Host-buffer entry: the batch is cut into row chunks (<= kHostChunks); chunk
 // i is copied in on s_in and, as soon as it has landed, the kernel computes the
 // output rows ending kHostLag rows above its last row (the rows it reads below
@@ -699,9 +726,25 @@ static perf_status host_enqueue(perf_plan_s* p, const void* host_in, void* host_
     const int n = (f1 - f0) * nc;
     for (int i = 0; i < n; ++i) {  // copy-in
       const int f = f0 + i / nc, c = i % nc, r0 = c * per, r1 = std::min(H, r0 + per);
-      const size_t off = (size_t)f * frame_bytes + (size_t)r0 * row_bytes;
-      CK(cudaMemcpyAsync(static_cast<char*>(p->d_stage_in) + off, static_cast<const char*>(host_in) + off,
-                         (size_t)(r1 - r0) * row_bytes, cudaMemcpyHostToDevice, p->s_in));
+      if (host_row_skip(p)) {
+        // row scheme: only the kept rows cross PCIe -- one strided 2-D copy per
+        // kept phase (the kernels never read a skipped row)
+        const int den = p->rate.den;
+        for (int ph = 0; ph < den; ++ph) {
+          if (!host_phase_kept(p, ph)) continue;
+          const int y0 = r0 + ((ph - r0) % den + den) % den;
+          if (y0 >= r1) continue;
+          const int cnt = (r1 - y0 + den - 1) / den;
+          const size_t off = (size_t)f * frame_bytes + (size_t)y0 * row_bytes;
+          CK(cudaMemcpy2DAsync(static_cast<char*>(p->d_stage_in) + off, den * row_bytes,
+                               static_cast<const char*>(host_in) + off, den * row_bytes, row_bytes, cnt,
+                               cudaMemcpyHostToDevice, p->s_in));
+        }
+      } else {
+        const size_t off = (size_t)f * frame_bytes + (size_t)r0 * row_bytes;
+        CK(cudaMemcpyAsync(static_cast<char*>(p->d_stage_in) + off, static_cast<const char*>(host_in) + off,
+                           (size_t)(r1 - r0) * row_bytes, cudaMemcpyHostToDevice, p->s_in));
+      }
       CK(cudaEventRecord(p->ev_in[i], p->s_in));
     }
     for (int i = 0; i < n; ++i) {  // compute + copy-out: output rows [r0, r1) lag the input chunk

@@ -158,3 +158,23 @@ def test_error_finish(metric, sums, want):
     PAPER.md:576-584 -- MRE and MAE divide by the count, ME by sum |e|"""
     with kp.Plan("gaussian", 8, 8, 2, metric=kp.METRIC[metric]) as p:
         assert kp.perf_error_finish(p.handle, sums) == want
+
+
+@pytest.mark.parametrize("scheme,rate,H,rows", [
+    ("row", (1, 2), 200, 100),   # Rows1: even rows
+    ("row", (3, 4), 202, 51),    # Rows2 (keep-one): rows = 0 mod 4
+    ("row", (1, 4), 202, 152),   # skip-one: rows = 3 mod 4 skipped (50 of them)
+    ("row", (0, 1), 202, 202),   # rate 0: exact
+    ("col", (1, 2), 202, 202),   # cells: whole rows cross PCIe
+])
+def test_host_h2d_bytes(scheme, rate, H, rows):
+    """PERF_KEY_H2D_BYTES (read-only): perf_run_host copies only the kept rows
+    of the row scheme host -> device (PERF_KEY_HOST_SKIP, default 1); host-only."""
+    W, B = 640, 2
+    with kp.Plan("gaussian", W, H, 2, scheme, rate, "li", batch=B) as p:
+        assert p.get("host_skip") == 1
+        assert p.get("h2d_bytes") == rows * W * 4 * B
+        p.set("host_skip", 0)
+        assert p.get("h2d_bytes") == H * W * 4 * B
+        with pytest.raises(kp.PerfError):
+            p.set("h2d_bytes", 1)

@@ -270,6 +270,42 @@ def test_run_host_pinned_pipeline(app, r, scheme, rate, recon, W, H, B):
         assert np.array_equal(pageable, want)
 
 
+@pytest.mark.parametrize("app,r,rate,recon,W,H", [
+    ("gaussian", 2, (1, 2), "li", 1024, 1030),
+    ("sobel", 1, (1, 4), "nn", 700, 517),
+    ("gauss_sobel", 2, (3, 4), "li", 520, 70),
+    ("median", 1, (1, 2), "nn", 2100, 300),
+])
+def test_run_host_skips_perforated_rows(app, r, rate, recon, W, H):
+    """Row scheme through perf_run_host: only the kept rows cross PCIe
+    (PERF_KEY_HOST_SKIP).  Skipped rows of the host input are poisoned (NaN /
+    0xFF) -- the output equals perf_run on the clean image bit for bit, with
+    and without the skip, so no skipped row is ever read (a1)."""
+    u8 = app == "median"
+    img = synth.image("natural", 61, W, H, np.uint8 if u8 else np.float32)
+    dev = torch.from_numpy(img).cuda()
+    want = torch.empty_like(dev)
+    num, den = rate
+    kept = [(y % den == 0) if num == den - 1 else (y % den != den - 1) for y in range(H)]
+    bad = img.copy()
+    for y in range(H):
+        if not kept[y]:
+            bad[y] = 255 if u8 else np.nan
+    with kp.Plan(app, W, H, r, "row", rate, recon) as p:
+        p.run(dev, want)
+        torch.cuda.synchronize()
+        want = want.cpu().numpy()
+        hin = torch.from_numpy(bad).pin_memory()
+        for skip in (1, 0):
+            p.set("host_skip", skip)
+            hout = torch.zeros_like(hin).pin_memory()
+            p.run_host(hin, hout)
+            assert np.array_equal(hout.numpy(), want), f"host_skip={skip}"
+        assert p.get("h2d_bytes") == H * W * img.itemsize  # (host_skip 0 now)
+        p.set("host_skip", 1)
+        assert p.get("h2d_bytes") == sum(kept) * W * img.itemsize
+
+
 def test_device_generator_matches_host():
     for cls in ("flat", "natural", "pattern"):
         d = torch.empty((2, 300, 500), dtype=torch.float32, device="cuda")
