@@ -893,8 +893,10 @@ cudaError_t launch_one(const KParams& p, unsigned grid, size_t smem, cudaStream_
   // segment boundary (halo + rebuild apron): KPERF_SEG_K1-row segments for them
   // (narrow 2-warp CTAs, C1's 512^2 frames: the row scheme keeps 64-row
   // segments -- Gaussian5 row 1/2 LI 135.6 us vs 145.6 with 16 rows)
+  // (radius-2 row scheme at den 2 -- Gaussian5 Rows1 -- measured best at 24)
   const int fseg = (SCHEME == S_ROW && NCW == 2) ? 64
-                   : (SCHEME == S_ROW && p.keep_one && p.den >= 4) ? KPERF_SEG_K1 : KPERF_SEG_FIX;
+                   : (SCHEME == S_ROW && p.keep_one && p.den >= 4) ? KPERF_SEG_K1
+                   : (SCHEME == S_ROW && p.den == 2 && App::VR == 2) ? KPERF_SEG_K1 : KPERF_SEG_FIX;
   const bool fixed64 = p.seg_auto && p.loader == L_BULK && App::VR <= 2 && App::NIN == 1 && sizeof(typename App::T) == 4 &&
                        SCHEME != S_STENCIL1 && fseg <= p.nrec - 2 * kMaxVR - kRecPad &&
                        (long long)p.n_strips * ((p.y_end - p.y_begin + fseg - 1) / fseg) * p.frames >= 2LL * n_sms;
