@@ -1,13 +1,14 @@
 """GPU <-> oracle parity in the EXACT launch configurations bench.py times.
 
 bench.py's C2 step is one perf_run over 8 frames of 4096^2 fp32 with 128-B
-cells; that batch is large enough for the launcher's fixed 64-row segments
-(kernel.cuh launch_one), which the small parity shapes never reach.  These
+cells; that batch is large enough for the launcher's fixed 16- / 24-row
+segments (kernel.cuh launch_one), which the small parity shapes never reach.  These
 tests build the bench's plans (same CONFIGS, batch, granule, seeds, device
 generator), run them once, and compare against oracle.run_pixels:
 
-* whole rows at and around every segment boundary the launcher can pick
-  (y = 0..2, 62..66, 126..130 and the last rows) on one frame;
+* whole rows at and around segment boundaries the launcher can pick
+  (y = 0..2, 14..18, 22..26, 46..50, 62..66, 126..130 and the last rows) on
+  one frame;
 * whole columns at and around the 1024-column strip boundaries (x = 1022..1026)
   and the image's right edge on another frame -- every row, so every segment
   boundary of any segment height is crossed;
@@ -50,7 +51,7 @@ def _frames(cfg, B):
 
 def _boundary_rows(H):
     ys = {0, 1, 2, H - 3, H - 2, H - 1}
-    for b in (64, 128):
+    for b in (16, 24, 48, 64, 128):  # fixed 16 / 24-row segments, wave-filling heights
         ys |= {b - 2, b - 1, b, b + 1, b + 2}
     ys |= {H // 2 - 1, H // 2}
     return sorted(y for y in ys if 0 <= y < H)
