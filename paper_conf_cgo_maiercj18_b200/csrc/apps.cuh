@@ -26,6 +26,9 @@
 #ifndef KPERF_FOLD_EDGE
 #define KPERF_FOLD_EDGE 1  // Gaussian / Sobel: the frame's first / last segments fold too (kernel.cuh)
 #endif
+#ifndef KPERF_GS_IPROD
+#define KPERF_GS_IPROD 0
+#endif
 #ifndef KPERF_GS_FOLD_ROT
 #define KPERF_GS_FOLD_ROT 1  // folded C5 loop: one kept row per iteration, register ring shifted (I-cache)
 #endif
@@ -356,7 +359,7 @@ struct AppHotspot {
 struct AppGaussSobel {
   using T = float;
   static constexpr bool ULI = KPERF_GS_ULI;  // uniform row LI (engine.cuh rebuild_frag)
-  static constexpr bool IPROD = false;  // PERF_KEY_PRODUCER 2 ignored: a smaller consumer loop (I-cache)
+  static constexpr bool IPROD = KPERF_GS_IPROD;  // 0: PERF_KEY_PRODUCER 2 ignored (a smaller consumer loop, I-cache)
   static constexpr int V = 8, EW = 4, VR = 3, NIN = 1, NWIN = 4, MINB = KPERF_GS_MINB;
   f2 acc[4][V / 2];  // Gaussian rows in flight (x 256), lane columns, pairs; slot q % 4
   float acce[4];     // the same for the lane's edge column (xc - 1 / xc + V)

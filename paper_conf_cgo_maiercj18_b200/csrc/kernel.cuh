@@ -669,6 +669,9 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
               wait = release = J <= Je;
             }
             if (App::FOLD_ROT || J <= Je) {
+              if constexpr (App::IPROD) {  // inline producer: make sure this row is issued
+                if (issuer && wait) issue_ahead(gi - g0);
+              }
               if (wait) mbar_wait_u32(full_u32 + 8 * (gi & nmask), (gi >> p.nr_log2) & 1);
               const float* row = ringf + (gi & nmask) * slot_elems;
               const Frag<float, V> c = ldf<float, V>(row + ccol);
