@@ -762,7 +762,7 @@ __device__ __noinline__ void consumer_generic(const KParams& p, const Mask& m, c
 // One work item per CTA: CTA b processes item b = (frame, segment of seg_h
 // output rows, strip of TW columns), strip fastest (the launcher sizes seg_h).
 template <class App, int SCHEME, int RECON, int NCW>
-__global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : (NCW == 2 ? 6 : App::MINB))
+__global__ void __launch_bounds__(32 * (NCW + 1), KPERF_MINB ? KPERF_MINB : (NCW == 2 ? 6 : (NCW == 3 ? 4 : App::MINB)))
     perf_kernel(const __grid_constant__ KParams p, const __grid_constant__ CUtensorMap tmap) {
   // (the TMA descriptor is a kernel parameter of its own: its generic address,
   // taken here, is what cp.async.bulk.tensor needs -- KParams::tmap is the host copy)
@@ -972,6 +972,10 @@ cudaError_t launch_sobel2(int, int, const KParams&, unsigned, size_t, cudaStream
 cudaError_t launch_median(int, int, const KParams&, unsigned, size_t, cudaStream_t);
 cudaError_t launch_hotspot(int, int, const KParams&, unsigned, size_t, cudaStream_t);
 cudaError_t launch_gsobel(int, int, const KParams&, unsigned, size_t, cudaStream_t);
+// fused pipeline on widths that are whole 768- but not 1024-column strips (C5's
+// 3840): CTAs of 3 consumer warps (+ producer), 4 per SM -- no idle warp in a
+// partial last strip
+cudaError_t launch_gsobel_n3(int, int, const KParams&, unsigned, size_t, cudaStream_t);
 cudaError_t launch_inversion(int, int, const KParams&, unsigned, size_t, cudaStream_t);
 
 constexpr int kNCW = 4;  // consumer warps per CTA (tile width 1024 fp32 / 4096 u8 columns)

@@ -139,6 +139,9 @@ static void hotspot_coeffs(float& sdc, float& rx1, float& ry1, float& rz1, float
   amb = 80.0f;
 }
 
+#ifndef KPERF_GS_NCW3
+#define KPERF_GS_NCW3 1  // fused pipeline: 3-warp CTAs on whole 768-column strips (make_params)
+#endif
 #ifndef KPERF_TMA
 #define KPERF_TMA 1  // auto loader: column / keep-one checkerboard cells by one TMA tensor-tile load per row
 #endif
@@ -198,7 +201,9 @@ static perf_status make_params(const perf_plan_s* P, const void* in, const void*
   const int V = P->app == PERF_APP_MEDIAN ? 16 : 8;
   // consumer warps per CTA: 2 for narrow fp32 Gaussian / Sobel images (kernel.cuh)
   const bool narrow = (P->app == PERF_APP_GAUSSIAN || P->app == PERF_APP_SOBEL) && P->W <= 2 * 32 * V;
-  const int NCW = narrow ? 2 : kp::kNCW;
+  // the fused pipeline on whole 768- but not 1024-column strips (C5's 3840): 3 (kernel.cuh)
+  const bool gs3 = KPERF_GS_NCW3 && P->app == PERF_APP_GAUSS_SOBEL && P->W % (3 * 32 * V) == 0 && P->W % (4 * 32 * V) != 0;
+  const int NCW = narrow ? 2 : (gs3 ? 3 : kp::kNCW);
   const int TW = NCW * 32 * V;
   const int Hg = P->global_h > 0 ? (int)P->global_h : P->H;
   int scheme = P->scheme;
@@ -389,7 +394,8 @@ static cudaError_t dispatch(const perf_plan_s* P, const KParams& k, unsigned gri
                             : kp::launch_sobel2(scheme, rc, k, grid, smem, s);
     case PERF_APP_MEDIAN: return kp::launch_median(scheme, rc, k, grid, smem, s);
     case PERF_APP_HOTSPOT: return kp::launch_hotspot(scheme, rc, k, grid, smem, s);
-    case PERF_APP_GAUSS_SOBEL: return kp::launch_gsobel(scheme, rc, k, grid, smem, s);
+    case PERF_APP_GAUSS_SOBEL:
+      return k.ncw == 3 ? kp::launch_gsobel_n3(scheme, rc, k, grid, smem, s) : kp::launch_gsobel(scheme, rc, k, grid, smem, s);
     case PERF_APP_INVERSION: return kp::launch_inversion(scheme, rc, k, grid, smem, s);
   }
   return cudaErrorInvalidValue;

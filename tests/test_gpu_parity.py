@@ -306,6 +306,19 @@ def test_run_host_skips_perforated_rows(app, r, rate, recon, W, H):
         assert p.get("h2d_bytes") == sum(kept) * W * img.itemsize
 
 
+@pytest.mark.parametrize("scheme,rate,recon", [("none", (0, 1), "nn"), ("row", (1, 2), "li"), ("row", (3, 4), "nn"),
+                                                ("col", (1, 2), "li"), ("checker", (3, 4), "nn")])
+def test_gauss_sobel_three_warp_ctas(scheme, rate, recon):
+    """The fused pipeline on whole 768- but not 1024-column strips (C5's 3840)
+    runs CTAs of 3 consumer warps (kperf.cu make_params): W = 1536 (two
+    strips), ragged segments, against the oracle."""
+    W, H = 1536, 150
+    img = synth.image("natural", 71, W, H)
+    got = gpu_run("gauss_sobel", 2, img, scheme, rate, recon, G_bytes=128)
+    want = oracle.run(oracle.params("gauss_sobel", W, H, 2, scheme, rate, recon, granule=32), img)
+    assert_close("gauss_sobel", 2, got, want)
+
+
 def test_device_generator_matches_host():
     for cls in ("flat", "natural", "pattern"):
         d = torch.empty((2, 300, 500), dtype=torch.float32, device="cuda")
