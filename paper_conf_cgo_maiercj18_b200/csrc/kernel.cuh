@@ -18,7 +18,7 @@
 #define KPERF_MINB 0  // 0: per-app App::MINB
 #endif
 #ifndef KPERF_SEG_K1
-#define KPERF_SEG_K1 24  // fixed segment height of keep-one row schemes with den >= 4 (see launch_one)
+#define KPERF_SEG_K1 24  // fixed segment height: keep-one row schemes with den >= 4, Gaussian5 row den 2 (launch_one)
 #endif
 #ifndef KPERF_SEG_FIX
 #define KPERF_SEG_FIX 16  // fixed segment height of the other fp32 whole-row kernels (see launch_one)
@@ -900,10 +900,10 @@ cudaError_t launch_one(const KParams& p, unsigned grid, size_t smem, cudaStream_
   const int fseg = (SCHEME == S_ROW && NCW == 2) ? 64
                    : (SCHEME == S_ROW && p.keep_one && p.den >= 4) ? KPERF_SEG_K1
                    : (SCHEME == S_ROW && p.den == 2 && App::VR == 2) ? KPERF_SEG_K1 : KPERF_SEG_FIX;
-  const bool fixed64 = p.seg_auto && p.loader == L_BULK && App::VR <= 2 && App::NIN == 1 && sizeof(typename App::T) == 4 &&
+  const bool fixed_seg = p.seg_auto && p.loader == L_BULK && App::VR <= 2 && App::NIN == 1 && sizeof(typename App::T) == 4 &&
                        SCHEME != S_STENCIL1 && fseg <= p.nrec - 2 * kMaxVR - kRecPad &&
                        (long long)p.n_strips * ((p.y_end - p.y_begin + fseg - 1) / fseg) * p.frames >= 2LL * n_sms;
-  if (fixed64) {
+  if (fixed_seg) {
     q.seg_h = fseg;
     q.n_segs = (p.y_end - p.y_begin + fseg - 1) / fseg;
     grid = (unsigned)((long long)q.n_strips * q.n_segs * q.frames);
