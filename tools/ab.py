@@ -32,6 +32,8 @@ SETS["colchk"] = [("gaussian", 2, "col", 1, 2, "li"), ("gaussian", 2, "col", 1, 
                   ("gaussian", 2, "checker", 3, 4, "li"), ("gaussian", 2, "checker", 3, 4, "nn"),
                   ("sobel", 1, "col", 1, 2, "nn"), ("sobel", 1, "col", 1, 4, "li"), ("sobel", 1, "checker", 3, 4, "li"),
                   ("gaussian", 2, "none", 0, 1, "nn")]
+SETS["stencil1"] = [("gaussian", 2, "stencil1", 0, 1, "nn"), ("sobel", 1, "stencil1", 0, 1, "nn"),
+                    ("gaussian", 2, "none", 0, 1, "nn")]
 SETS["all"] = SETS["row"] + SETS["col"] + SETS["checker"]
 
 CHILD = r'''
