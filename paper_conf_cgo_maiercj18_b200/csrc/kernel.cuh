@@ -894,14 +894,17 @@ cudaError_t launch_one(const KParams& p, unsigned grid, size_t smem, cudaStream_
   const int n_sms = dev_sms();
   // keep-one row schemes of den >= 4 re-read up to den - 1 extra kept rows per
   // segment boundary (halo + rebuild apron): KPERF_SEG_K1-row segments for them
-  // (narrow 2-warp CTAs, C1's 512^2 frames: the row scheme keeps 64-row
-  // segments -- Gaussian5 row 1/2 LI 135.6 us vs 145.6 with 16 rows)
+  // (narrow 2-warp CTAs, C1's 512^2 frames: the row scheme runs 32-row
+  // segments -- Gaussian5 row 1/2 LI 131.6 us vs 145.6 with 16, 135.3 with 64)
   // (radius-2 row scheme at den 2 -- Gaussian5 Rows1 -- measured best at 24)
-  const int fseg = (SCHEME == S_ROW && NCW == 2) ? 64
+  // (Stencil1: whole tile rows, >= 16 rows: 174 -> 162 us on C2)
+  const int th1 = SCHEME == S_STENCIL1 ? p.tile1_h : 1;
+  const int fseg = (SCHEME == S_STENCIL1) ? (KPERF_SEG_FIX + th1 - 1) / th1 * th1
+                   : (SCHEME == S_ROW && NCW == 2) ? 32
                    : (SCHEME == S_ROW && p.keep_one && p.den >= 4) ? KPERF_SEG_K1
                    : (SCHEME == S_ROW && p.den == 2 && App::VR == 2) ? KPERF_SEG_K1 : KPERF_SEG_FIX;
   const bool fixed_seg = p.seg_auto && p.loader == L_BULK && App::VR <= 2 && App::NIN == 1 && sizeof(typename App::T) == 4 &&
-                       SCHEME != S_STENCIL1 && fseg <= p.nrec - 2 * kMaxVR - kRecPad &&
+                       fseg <= p.nrec - 2 * kMaxVR - kRecPad &&
                        (long long)p.n_strips * ((p.y_end - p.y_begin + fseg - 1) / fseg) * p.frames >= 2LL * n_sms;
   if (fixed_seg) {
     q.seg_h = fseg;
