@@ -392,6 +392,9 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
       const float* ringf = reinterpret_cast<const float*>(ring);
       auto chk = [&](auto nc, int gxm, int col) {
         constexpr int N = decltype(nc)::value;
+#ifdef KPERF_PROBE_NOREBUILD  // experiment (DESIGN "cell loaders"): own packed column only, no rebuild
+        if (p.y_begin != -12345) return ldf<float, N>(ringf + (yr & nmask) * slot_elems + col);
+#endif
         int t = gxm + ym;
         if (t >= m.den) t -= m.den;
         const int4 e = etab[t];
@@ -450,6 +453,9 @@ __device__ void consumer(const KParams& p, const Mask& m, const RowPlan& rp, int
       auto colrow = [&](auto nc, const ColF& z, int col, const float4* wt) {
         constexpr int N = decltype(nc)::value;
         const Frag<float, N> c = ldf<float, N>(row + col);
+#ifdef KPERF_PROBE_NOREBUILD  // experiment: own packed column only, no rebuild
+        if (p.y_begin != -12345) return c;
+#endif
         const float a = row[z.ca], b = row[z.cb];
         Frag<float, N> o;
         if constexpr (RECON == R_LI) {
