@@ -142,6 +142,9 @@ static void hotspot_coeffs(float& sdc, float& rx1, float& ry1, float& rz1, float
 #ifndef KPERF_GS_NCW3
 #define KPERF_GS_NCW3 1  // fused pipeline: 3-warp CTAs on whole 768-column strips (make_params)
 #endif
+#ifndef KPERF_TMA_PROMO
+#define KPERF_TMA_PROMO CU_TENSOR_MAP_L2_PROMOTION_L2_128B  // L2 promotion of the TMA cell tiles
+#endif
 #ifndef KPERF_TMA
 #define KPERF_TMA 1  // auto loader: column / keep-one checkerboard cells by one TMA tensor-tile load per row
 #endif
@@ -176,7 +179,7 @@ static bool encode_tma(KParams& k, const void* in, int W, long long rows) {
     const cuuint32_t box[3] = {(cuuint32_t)k.tma_L, (cuuint32_t)k.tma_ng, 1};
     const cuuint32_t es[3] = {1, 1, 1};
     r = enc(&k.tmap, CU_TENSOR_MAP_DATA_TYPE_FLOAT32, 3, const_cast<void*>(in), dims, strides, box, es,
-            CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_128B,
+            CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, KPERF_TMA_PROMO,
             CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
   } else {  // {G, cell, row}, traversal stride den along the cells: every den-th cell from the start cell
     const cuuint64_t dims[3] = {G, ng * den, (cuuint64_t)rows};
@@ -184,7 +187,7 @@ static bool encode_tma(KParams& k, const void* in, int W, long long rows) {
     const cuuint32_t box[3] = {(cuuint32_t)G, (cuuint32_t)(k.tma_ng * k.den), 1};
     const cuuint32_t es[3] = {1, (cuuint32_t)k.den, 1};
     r = enc(&k.tmap, CU_TENSOR_MAP_DATA_TYPE_FLOAT32, 3, const_cast<void*>(in), dims, strides, box, es,
-            CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, CU_TENSOR_MAP_L2_PROMOTION_L2_128B,
+            CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_NONE, KPERF_TMA_PROMO,
             CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
   }
   return r == CUDA_SUCCESS;
