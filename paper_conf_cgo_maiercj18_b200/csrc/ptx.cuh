@@ -51,12 +51,31 @@ __device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t parity) {
 }
 
 // TMA engine 1D bulk copy global -> shared, completion signalled as tx bytes on bar.
+#ifndef KPERF_LD_EVICT
+#define KPERF_LD_EVICT 0  // experiment: bulk row loads with an L2 evict-first cache policy
+#endif
+#ifndef KPERF_ST_EVICT
+#define KPERF_ST_EVICT 0  // experiment: 256-bit output stores with an L2 evict-first cache policy
+#endif
+__device__ __forceinline__ uint64_t l2_evict_first_policy() {
+  uint64_t pol;
+  asm volatile("createpolicy.fractional.L2::evict_first.b64 %0, 1.0;" : "=l"(pol));
+  return pol;
+}
 __device__ __forceinline__ void bulk_g2s(void* dst, const void* src, uint32_t bytes, uint64_t* bar) {
+#if KPERF_LD_EVICT
+  asm volatile(
+      "cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes.L2::cache_hint [%0], [%1], %2, [%3], %4;" ::"r"(
+          smem_u32(dst)),
+      "l"(src), "r"(bytes), "r"(smem_u32(bar)), "l"(l2_evict_first_policy())
+      : "memory");
+#else
   asm volatile(
       "cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(
           smem_u32(dst)),
       "l"(src), "r"(bytes), "r"(smem_u32(bar))
       : "memory");
+#endif
 }
 
 // TMA tensor tile loads (UTMALDG): box at the given coordinates of the tensor
@@ -110,9 +129,16 @@ __device__ __forceinline__ void st_global_v4(void* p, uint32_t a, uint32_t b, ui
 // a warp's row chunk (32 lanes x 32 B) is one fully coalesced 1-KB request;
 // two 128-bit stores per lane each wrote half of every 32-B sector.
 __device__ __forceinline__ void st_global_v8(void* p, const uint4& a, const uint4& b) {
+#if KPERF_ST_EVICT
+  asm volatile("st.global.L1::no_allocate.L2::cache_hint.v8.b32 [%0], {%1, %2, %3, %4, %5, %6, %7, %8}, %9;" ::"l"(p),
+               "r"(a.x), "r"(a.y), "r"(a.z), "r"(a.w), "r"(b.x), "r"(b.y), "r"(b.z), "r"(b.w),
+               "l"(l2_evict_first_policy())
+               : "memory");
+#else
   asm volatile("st.global.L1::no_allocate.v8.b32 [%0], {%1, %2, %3, %4, %5, %6, %7, %8};" ::"l"(p), "r"(a.x),
                "r"(a.y), "r"(a.z), "r"(a.w), "r"(b.x), "r"(b.y), "r"(b.z), "r"(b.w)
                : "memory");
+#endif
 }
 
 // packed fp16x2 min / max (HMNMX2).  Median lanes hold 0x6400|v (fp16 1024+v),
