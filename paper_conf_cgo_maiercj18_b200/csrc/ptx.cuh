@@ -52,7 +52,7 @@ __device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t parity) {
 
 // TMA engine 1D bulk copy global -> shared, completion signalled as tx bytes on bar.
 #ifndef KPERF_LD_EVICT
-#define KPERF_LD_EVICT 0  // experiment: bulk row loads with an L2 evict-first cache policy
+#define KPERF_LD_EVICT 2  // bulk row loads: L2 evict-first (1, slower: halo rows re-read) / evict-last (2, default: +0.5-1%) / none (0)
 #endif
 #ifndef KPERF_ST_EVICT
 #define KPERF_ST_EVICT 0  // experiment: 256-bit output stores with an L2 evict-first cache policy
@@ -62,12 +62,17 @@ __device__ __forceinline__ uint64_t l2_evict_first_policy() {
   asm volatile("createpolicy.fractional.L2::evict_first.b64 %0, 1.0;" : "=l"(pol));
   return pol;
 }
+__device__ __forceinline__ uint64_t l2_evict_last_policy() {
+  uint64_t pol;
+  asm volatile("createpolicy.fractional.L2::evict_last.b64 %0, 1.0;" : "=l"(pol));
+  return pol;
+}
 __device__ __forceinline__ void bulk_g2s(void* dst, const void* src, uint32_t bytes, uint64_t* bar) {
 #if KPERF_LD_EVICT
   asm volatile(
       "cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes.L2::cache_hint [%0], [%1], %2, [%3], %4;" ::"r"(
           smem_u32(dst)),
-      "l"(src), "r"(bytes), "r"(smem_u32(bar)), "l"(l2_evict_first_policy())
+      "l"(src), "r"(bytes), "r"(smem_u32(bar)), "l"(KPERF_LD_EVICT == 2 ? l2_evict_last_policy() : l2_evict_first_policy())
       : "memory");
 #else
   asm volatile(
